@@ -75,7 +75,7 @@ def test_dataset_size_footnote2():
     # fn. 2: each parameter counted once even if inout: matmul fp32 b=256 -> 786432 B.
     m, _ = _matmul_model(1, b=256)
     assert m.dataset_size(m.tasks[0]) == 786432
-    m2, _ = _chol_model(2, b=512)
+    m2, _ = _chol_model(3, b=512)
     sizes = sorted({(m2.types[t["type"]][0], m2.dataset_size(t)) for t in m2.tasks})
     assert sizes == [("GEMM_NT", 3 << 20), ("POTRF", 1 << 20), ("SYRK", 2 << 20), ("TRSM", 2 << 20)]
 
