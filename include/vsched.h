@@ -1,0 +1,274 @@
+/*
+ * vsched.h — C ABI of libvsched: self-adaptive versioned tile tasks on B200.
+ *
+ * The calls follow the problem statement of Planas, Badia, Ayguade, Labarta,
+ * "Self-Adaptive OmpSs Tasks in Heterogeneous Environments", IPDPS 2013
+ * (PAPER.md line numbers L..., section in parentheses):
+ *   - task functions with input/output/inout data (L231-242, Sec III)
+ *   - several implementations of one task, "implements(main)"
+ *     (L270-276, L298-351, Sec IV.A, Fig 4)
+ *   - copy_deps data motion between address spaces (L220-230, L252-264)
+ *   - taskwait / taskwait on / noflush (L243-246, L264-270)
+ *   - scheduler plug-in and its options chosen by configuration (L277-288);
+ *     lambda configurable (L438-440, footnote 4 L461)
+ *   - versioning scheduler: TaskVersionSet <VersionId, ExecTime, #Exec> per
+ *     DataSetSize group (L358-385, Table I), learning phase then earliest
+ *     executor (L397-495, Fig 5)
+ *   - statistics: Input/Output/Device Tx and per-version run counts (L515-536)
+ * Readings where the paper is silent are numbered R1..R25 in DESIGN.md.
+ *
+ * Conventions
+ *   - Every function returns vs_status (0 = VS_OK, negative = error) unless
+ *     stated.  Synchronous misuse returns an error and sets vs_last_error().
+ *   - Asynchronous failures (CUDA error, non-positive Cholesky pivot) are
+ *     STICKY: they are returned by the next vs_wait_* call; afterwards only
+ *     vs_stats*, vs_last_error and vs_destroy are valid.
+ *   - Pointers passed as task data are NOT owned by the runtime.  The caller
+ *     must not touch registered data between the submission of a task that
+ *     uses it and the wait that covers it (OmpSs rule, L264-270).
+ *   - "stream" arguments are cudaStream_t passed as void* (NULL = legacy
+ *     default stream); no CUDA or torch type appears in this header.
+ *   - Single submitting thread (OmpSs master-thread model, L213-215).
+ */
+#ifndef VSCHED_H
+#define VSCHED_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+#if defined(__GNUC__)
+#pragma GCC visibility push(default)
+#endif
+
+typedef struct vs_runtime *vs_rt;
+typedef int32_t vs_type_id;
+typedef int32_t vs_version_id;
+typedef int64_t vs_data_id;
+typedef int64_t vs_task_id;
+
+/* Access modes of a task parameter (StarSs clauses, L236-242). */
+enum { VS_IN = 1, VS_OUT = 2, VS_INOUT = 3 };
+
+typedef enum {
+    VS_OK = 0,
+    VS_E_INVAL = -1,     /* bad argument / unknown id */
+    VS_E_NOMEM = -2,     /* host or device allocation failed */
+    VS_E_CUDA = -3,      /* CUDA error (sticky when asynchronous) */
+    VS_E_NOT_SPD = -4,   /* potrf found a non-positive pivot (sticky, R9) */
+    VS_E_STATE = -5,     /* call not valid in the current state (e.g. after a sticky error) */
+    VS_E_OVERLAP = -6,   /* registered regions partially overlap (R21) */
+    VS_E_NODEV = -7,     /* no CUDA device / library built without a usable device */
+    VS_E_IO = -8         /* timing-table file could not be read or written */
+} vs_status;
+
+/* Executors. */
+enum { VS_EXEC_GPU = 0, /* tasks run on B200s */
+       VS_EXEC_SIM = 1  /* no device: tasks take their durations from the timing
+                           table on a virtual clock (DES); used for replay tests */ };
+/* When a decision is taken (GPU executor). */
+enum { VS_MODE_RUNAHEAD = 0, /* decide on the virtual clock as soon as predecessors are
+                                decided; dependences are enforced on the device
+                                ("look-ahead scheduling", L811) — default */
+       VS_MODE_READY = 1     /* paper-literal: decide when predecessors have really
+                                completed (L400-405) */ };
+enum { VS_LEARN_HOLD = 0, VS_LEARN_RR = 1 };            /* reading R12 */
+enum { VS_POLICY_VERSIONING = 0, VS_POLICY_FIXED = 1 };  /* FIXED = always fixed_version */
+enum { VS_F32 = 0, VS_F64 = 1 };
+
+/* Built-in tile task types (reading R5).  Tiles are b x b,
+ * row-major, contiguous (leading dimension b), D6.  Parameters in order:
+ *   VS_T_MATMUL : in A, in B, inout C        C += A * B            (Fig 1)
+ *   VS_T_POTRF  : inout A                    A  = L, L*L^T = A     (lower, in place; L697-699)
+ *   VS_T_TRSM   : in L, inout B              B  = B * L^{-T}       (right, lower, trans, non-unit)
+ *   VS_T_SYRK   : in A, inout C              C -= A * A^T          (lower triangle only)
+ *   VS_T_GEMM_NT: in A, in B, inout C        C -= A * B^T
+ * The strict upper triangle of POTRF/SYRK tiles is neither read nor written (R7). */
+enum { VS_T_MATMUL = 0, VS_T_POTRF = 1, VS_T_TRSM = 2, VS_T_SYRK = 3, VS_T_GEMM_NT = 4,
+       VS_NUM_BUILTIN_TYPES = 5 };
+
+/* Built-in versions (hand-written sm_100a kernels; "implements(main)" siblings). */
+enum {
+    VS_V_SIMT_F32 = 0,    /* IEEE fp32 FMA, fixed ascending-k order, smem staging + warp shuffles */
+    VS_V_TC_3XTF32 = 1,   /* tcgen05/TMEM 3xTF32 (big*big + big*small + small*big) */
+    VS_V_F64IN_F32IO = 2, /* fp32 in/out, fp64 arithmetic (DMMA), one rounding on store */
+    VS_V_DFMA_F64 = 3,    /* fp64 tiles, SIMT DFMA */
+    VS_V_DMMA_F64 = 4,    /* fp64 tiles, mma.sync f64 tensor cores */
+    VS_NUM_BUILTIN_VERSIONS = 5
+};
+
+typedef struct {
+    int exec;          /* VS_EXEC_GPU | VS_EXEC_SIM */
+    int n_gpus;        /* number of devices driven by this runtime (workers' gpus 0..n_gpus-1) */
+    int device_base;   /* CUDA ordinal of runtime gpu 0 (one process per GPU: LOCAL_RANK) */
+    int slots_per_gpu; /* S workers (streams) per GPU (R16); S=1 is paper-literal */
+    int lambda;        /* learning runs per version (L438-440, L461); default 3 (R10) */
+    int policy;        /* VS_POLICY_VERSIONING | VS_POLICY_FIXED */
+    int fixed_version; /* version index used by VS_POLICY_FIXED */
+    int learning;      /* VS_LEARN_HOLD | VS_LEARN_RR */
+    int mode;          /* VS_MODE_RUNAHEAD | VS_MODE_READY */
+    int replay;        /* 1: the scheduler takes run times from the timing table, not from
+                          measurements (bit-exact decisions, P8).  Implied by VS_EXEC_SIM. */
+    int flush;         /* 1 (default): vs_wait_all copies written data back to its home
+                          (OmpSs flush, L264-270) */
+} vs_config;
+
+/* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,
+ * run-ahead, live timing, flush.  Environment overrides applied by vs_create (L277-288):
+ * VS_LAMBDA, VS_SLOTS, VS_POLICY(=versioning|fixed:<v>), VS_LEARNING(=hold|rr),
+ * VS_MODE(=runahead|ready). */
+void vs_config_default(vs_config *cfg);
+
+/* Create a runtime.  *out receives an opaque handle owning scheduler state, DAG,
+ * data directory, CUDA streams/events and device replicas.
+ * Errors: VS_E_INVAL (bad cfg), VS_E_NODEV (exec GPU but no device), VS_E_CUDA. */
+int vs_create(const vs_config *cfg, vs_rt *out);
+/* Wait for all tasks (no flush), release every resource.  Safe after a sticky error. */
+int vs_destroy(vs_rt rt);
+/* Last error message of this runtime (static storage until the next call); never NULL. */
+const char *vs_last_error(vs_rt rt);
+
+/* ---------------------------------------------------------- registration (a1) */
+/* Declare a task type ("main implementation", L298-351) with nparams parameters
+ * whose access modes are modes[i] in {VS_IN, VS_OUT, VS_INOUT}. */
+int vs_type_create(vs_rt rt, const char *name, int nparams, const int *modes, vs_type_id *out);
+
+/* A version launch function: enqueue the version's work for one task on `stream`
+ * (a cudaStream_t).  dev_ptrs[i] is parameter i on the executing GPU, bytes[i] its
+ * size.  Must not synchronise the stream, must touch only its parameters, must be
+ * deterministic.  Return 0 on success. */
+typedef int (*vs_launch_fn)(void *const *dev_ptrs, const int64_t *bytes, int nargs,
+                            const void *scalars, size_t nscalar, void *stream, void *user);
+
+/* Add a version to a type ("implements(main)", Fig 4).  All versions share the
+ * type's parameters and modes (L306-308).  gpu_mask bit g = runnable on runtime gpu g
+ * (the device clause, L339-345).  *out = version index within the type (0,1,...). */
+int vs_version_add(vs_rt rt, vs_type_id type, const char *name, uint32_t gpu_mask,
+                   vs_launch_fn fn, void *user, vs_version_id *out);
+
+/* Register the five built-in tile task types for dtype (VS_F32: versions SIMT_F32,
+ * TC_3XTF32, F64IN_F32IO; VS_F64: DFMA_F64, DMMA_F64), keeping the versions whose
+ * bit is set in version_mask (bit = VS_V_*).  out_types[VS_T_*] receives the type ids;
+ * version index order inside each type follows increasing VS_V_* id.  Runnable on
+ * every gpu.  Errors: VS_E_INVAL if no version of dtype is selected. */
+int vs_register_builtins(vs_rt rt, int dtype, uint32_t version_mask,
+                         vs_type_id out_types[VS_NUM_BUILTIN_TYPES]);
+
+/* ------------------------------------------------------------ data (a2, a8) */
+/* Register a datum (a tile) living at ptr in the memory of `device` (-1 = host,
+ * preferably pinned; g >= 0 = runtime gpu g).  Identical (ptr, bytes) returns the
+ * same id; a partial overlap with a registered region is VS_E_OVERLAP (R21). */
+int vs_data_register(vs_rt rt, void *ptr, int device, int64_t bytes, vs_data_id *out);
+
+/* ------------------------------------------------------------- submission (a2) */
+/* Create a task instance: RAW/WAR/WAW edges on whole data (L236-242).  scalars
+ * (may be NULL) are copied and passed to the version.  Execution happens inside
+ * the vs_wait_* calls (the submitting thread joins the runtime, as at taskwait). */
+int vs_submit(vs_rt rt, vs_type_id type, const vs_data_id *args, int nargs,
+              const void *scalars, size_t nscalar, vs_task_id *out);
+
+/* ----------------------------------------------------------- waits (a15) */
+int vs_wait_all(vs_rt rt);          /* taskwait: all tasks, then flush to home */
+int vs_wait_all_noflush(vs_rt rt);  /* taskwait noflush (L267-270) */
+int vs_wait_on(vs_rt rt, vs_data_id d); /* taskwait on(d): d's last writer done; d valid at home */
+
+/* ---------------------------------------------------------------- statistics */
+typedef struct {
+    int64_t tasks_submitted, tasks_completed, decisions;
+    int64_t input_tx_bytes;   /* host -> any GPU, counted per destination (L529-532, R25) */
+    int64_t output_tx_bytes;  /* any GPU -> host (L527-528) */
+    int64_t device_tx_bytes;  /* GPU <-> GPU (L524-525) */
+    int64_t n_groups;
+    int64_t error_task;       /* task of the first sticky error, -1 if none */
+    int64_t error_info;       /* potrf info (1-based pivot within the tile), or CUDA error code */
+    int64_t host_ns_decide;   /* host time spent in decisions (scheduler overhead) */
+    int64_t host_ns_issue;    /* host time spent issuing GPU work */
+    int64_t virtual_now_ns;   /* DES clock */
+} vs_stats_t;
+int vs_stats(vs_rt rt, vs_stats_t *out);
+
+#define VS_MAX_VERSIONS 8
+typedef struct {
+    vs_type_id type;
+    int64_t dataset_bytes;             /* DataSetSize (footnote 2) */
+    int nversions;
+    int reliable;                      /* 1 once every runnable version ran lambda times */
+    int64_t first_reliable_decision;   /* 1-based decision index within the group, -1 if none */
+    int64_t decisions;
+    int64_t n[VS_MAX_VERSIONS];        /* #Exec (completed, measured) */
+    int64_t mean_ns[VS_MAX_VERSIONS];  /* ExecTime = floor(sum/n) (R18), 0 if n = 0 */
+    int64_t assigned[VS_MAX_VERSIONS]; /* decisions that picked this version */
+} vs_group_stat_t;
+int vs_group_count(vs_rt rt);
+int vs_group_stat(vs_rt rt, int group_index, vs_group_stat_t *out);
+/* Name of a type / of version v of a type (static storage owned by rt); NULL if invalid. */
+const char *vs_type_name(vs_rt rt, vs_type_id t);
+const char *vs_version_name(vs_rt rt, vs_type_id t, vs_version_id v);
+
+/* Decision log: one record per decision, in decision order. */
+typedef struct {
+    vs_task_id task;
+    int32_t version, worker;   /* worker = gpu * slots_per_gpu + slot */
+    int32_t phase, pad;        /* 0 learning, 1 reliable */
+    int64_t t_decide_ns;       /* virtual (run-ahead / sim) or host clock (ready) */
+    int64_t t_start_ns, t_end_ns; /* sim: virtual; gpu: measured start/end (0 if unknown) */
+} vs_decision_t;
+/* Copy up to cap records (from the beginning) into out; *n = total records. */
+int vs_decision_log(vs_rt rt, vs_decision_t *out, int64_t cap, int64_t *n);
+/* FNV-1a 64 over (task, version, worker, t_decide) of every record, little-endian int64
+ * (identical definition in oracle/sched_model.py). */
+uint64_t vs_decision_log_hash(vs_rt rt);
+int vs_decision_log_clear(vs_rt rt);
+
+/* ---------------------------------------------------- timing table (NEXT-2) */
+/* Text format, one line per (type, group, version):
+ *   <type name> <dataset bytes> <version name> <mean ns> <n>
+ * dump writes the current TaskVersionSets; load merges (sum = mean*n, assigned = n)
+ * and switches loaded groups to reliable when every runnable version has n >= lambda. */
+int vs_table_dump(vs_rt rt, const char *path);
+int vs_table_load(vs_rt rt, const char *path);
+/* Replay/sim duration of (type, dataset bytes, version); used when exec = SIM or
+ * replay = 1.  A missing entry during replay is VS_E_STATE. */
+int vs_replay_set(vs_rt rt, vs_type_id type, int64_t dataset_bytes, vs_version_id v, int64_t ns);
+
+/* ---------------------------------------------- application drivers (Fig 1, R5) */
+/* Tiled matmul driver of Fig 1 (L164-172): for i<m, j<n, k<l submit
+ * MATMUL(A[i*l+k], B[k*n+j], C[i*n+j]).  A, B, C are arrays of data ids. */
+int vs_app_matmul(vs_rt rt, vs_type_id matmul_type, int m, int l, int n,
+                  const vs_data_id *A, const vs_data_id *B, const vs_data_id *C);
+/* Right-looking lower tiled Cholesky (R5): A[i*nt+j] for i >= j, types[VS_T_*]. */
+int vs_app_cholesky(vs_rt rt, const vs_type_id types[VS_NUM_BUILTIN_TYPES], int nt,
+                    const vs_data_id *A);
+
+/* ----------------------------------------------------- direct tile kernels */
+/* Enqueue one built-in tile task version on `stream` on the current device, outside
+ * the runtime (used by parity tests and the smoke check).  ptrs as in VS_T_* order,
+ * device pointers, tiles b x b contiguous.  dinfo: device int32 receiving potrf's info
+ * (may be NULL for other types).  Returns VS_E_INVAL for an unknown (type, version)
+ * or an unsupported b (b must be a multiple of 32, 32 <= b <= 4096). */
+int vs_tile_run(int type, int version, int b, void *const *ptrs, int *dinfo, void *stream);
+
+/* ---------------------------------------------------------- input generator */
+/* Device counter-based generator, bit-identical to vsgen.uniform_idx:
+ *   u(seed, idx) = (splitmix64((seed << 40) | idx) >> 40) * 2^-23 - 1.
+ * Writes a rows x cols matrix (global index r*cols+c) as dtype VS_F32/VS_F64 into
+ * dev_out: row-major if tile_b == 0, else tile-major (tiles tile_b x tile_b row-major,
+ * tile (I,J) at offset (I*(cols/tile_b)+J)*tile_b^2). */
+int vs_gen_uniform(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b,
+                   void *dev_out, void *stream);
+/* SPD recipe R8: S_rc = u(seed, max(r,c)*n + min(r,c)); diagonal fl(S_rr + alpha) with
+ * alpha = 2.5*sqrt(n) (n >= 256) else n, computed in fp64.  Layout as vs_gen_uniform. */
+int vs_gen_spd(uint64_t seed, int64_t n, int dtype, int tile_b, void *dev_out, void *stream);
+
+/* Library build information (never NULL). */
+const char *vs_build_info(void);
+
+#if defined(__GNUC__)
+#pragma GCC visibility pop
+#endif
+#ifdef __cplusplus
+}
+#endif
+#endif /* VSCHED_H */

@@ -1,0 +1,20 @@
+// kernels.hpp — internal interface between the runtime and the sm_100a tile kernels.
+// Not part of the public ABI (see include/vsched.h).
+#pragma once
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+namespace vsk {
+
+// Task types / versions use the VS_T_* / VS_V_* numbering of vsched.h.
+// Returns 0 on success, -1 for an unsupported (type, version, b).
+int launch_builtin(int type, int version, int b, void *const *p, int *dinfo, cudaStream_t s);
+bool builtin_supported(int type, int version, int b);
+// Element size in bytes for a version (4 for f32-io versions, 8 for f64).
+int builtin_elem_bytes(int version);
+
+int gen_uniform(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b, void *out,
+                cudaStream_t s);
+int gen_spd(uint64_t seed, int64_t n, int dtype, int tile_b, void *out, cudaStream_t s);
+
+}  // namespace vsk

@@ -1,0 +1,379 @@
+// tc_gemm.cuh — tcgen05 / TMEM 3xTF32 tile GEMM (version tc_3xtf32), sm_100a.
+//
+//   C[M x N] (ldc) = C + s * A[M x K] (lda) * op(B),  s = +1 (matmul) or -1 (Cholesky
+//   gemm / syrk / trsm / potrf updates), op(B) = B (NN) or B^T (NT).
+//
+// 3xTF32: every fp32 operand x is split into big = rna_tf32(x) and small = x - big
+// (exact in fp32), and D += Ab*Bb + Ab*Bs + As*Bb is accumulated in fp32 in TMEM by
+// three tcgen05.mma.kind::tf32 per k-step (the dropped As*Bs term is < 2^-22 |a||b|).
+//
+// Structure (one 128 x BN output tile per CTA, cta_group::1):
+//   warps 0-3  producers: LDG.128 fp32 k-blocks (32 wide) -> split in registers ->
+//              STS into 128B-swizzled K-major (A, and B in NT form) or MN-major (B in
+//              NN form) UMMA layouts; fence.proxy.async; mbarrier arrive (full[s]).
+//              The next k-block's loads are in flight while the current one is stored.
+//   warp 4     TMEM allocator + MMA issuer: one elected lane waits full[s], issues
+//              3 x (BK/8) MMAs, tcgen05.commit -> empty[s]; after the last k-block,
+//              commit -> acc_full.
+//   warps 0-3  epilogue: tcgen05.ld 32x32b.x32 (warp w owns TMEM lanes 32w..32w+31 =
+//              tile rows), C += acc with fp32 round-to-nearest, vector stores.
+// LOWER (syrk / potrf update): CTAs strictly above the diagonal exit; diagonal tiles
+// store only j <= i.
+#pragma once
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+namespace vsk {
+namespace tc {
+
+constexpr int BM = 128, BK = 32, STAGES = 3;
+constexpr int NPROD = 128;  // producer / epilogue threads (warps 0-3)
+constexpr int NTHREADS = NPROD + 32;
+
+__device__ __forceinline__ uint32_t smem_u32(const void *p) { return (uint32_t)__cvta_generic_to_shared(p); }
+
+__device__ __forceinline__ void mbar_init(uint64_t *bar, uint32_t count)
+{
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
+}
+__device__ __forceinline__ void mbar_arrive(uint64_t *bar)
+{
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t *bar, uint32_t parity)
+{
+    asm volatile(
+        "{\n\t.reg .pred P1;\n"
+        "WAIT_%=:\n\t"
+        "mbarrier.try_wait.parity.shared::cta.b64 P1, [%0], %1;\n\t"
+        "@P1 bra DONE_%=;\n\t"
+        "bra WAIT_%=;\n"
+        "DONE_%=:\n\t}" ::"r"(smem_u32(bar)),
+        "r"(parity)
+        : "memory");
+}
+__device__ __forceinline__ void fence_proxy_async() { asm volatile("fence.proxy.async.shared::cta;" ::: "memory"); }
+__device__ __forceinline__ void tc_fence_before() { asm volatile("tcgen05.fence::before_thread_sync;" ::: "memory"); }
+__device__ __forceinline__ void tc_fence_after() { asm volatile("tcgen05.fence::after_thread_sync;" ::: "memory"); }
+
+__device__ __forceinline__ float to_tf32(float x)
+{
+    uint32_t r;
+    asm("cvt.rna.tf32.f32 %0, %1;" : "=r"(r) : "f"(x));
+    return __uint_as_float(r);
+}
+
+// UMMA shared-memory descriptor (sm_100): start>>4 [0,14), LBO>>4 [16,30), SBO>>4 [32,46),
+// version=1 [46,48), base offset 0, layout SWIZZLE_128B = 2 at [61,64).
+__device__ __forceinline__ uint64_t make_desc(uint32_t saddr, uint32_t lbo, uint32_t sbo)
+{
+    uint64_t d = 0;
+    d |= (uint64_t)((saddr & 0x3FFFF) >> 4);
+    d |= (uint64_t)((lbo >> 4) & 0x3FFF) << 16;
+    d |= (uint64_t)((sbo >> 4) & 0x3FFF) << 32;
+    d |= (uint64_t)1 << 46;
+    d |= (uint64_t)2 << 61;
+    return d;
+}
+
+// Instruction descriptor, kind::tf32: D f32 (bit 4), A/B tf32 (=2 at bits 7, 10),
+// negate A (bit 13), B major (bit 16: 1 = MN-major), N>>3 at 17, M>>4 at 24.
+__host__ __device__ constexpr uint32_t make_idesc(int M, int N, bool negA, bool b_mn_major)
+{
+    return (1u << 4) | (2u << 7) | (2u << 10) | ((negA ? 1u : 0u) << 13) | ((b_mn_major ? 1u : 0u) << 16) |
+           ((uint32_t)(N >> 3) << 17) | ((uint32_t)(M >> 4) << 24);
+}
+
+__device__ __forceinline__ void mma_tf32(uint32_t tmem_d, uint64_t adesc, uint64_t bdesc, uint32_t idesc, uint32_t acc)
+{
+    asm volatile(
+        "{\n\t.reg .pred p;\n\t"
+        "setp.ne.b32 p, %4, 0;\n\t"
+        "tcgen05.mma.cta_group::1.kind::tf32 [%0], %1, %2, %3, p;\n\t}" ::"r"(tmem_d),
+        "l"(adesc), "l"(bdesc), "r"(idesc), "r"(acc));
+}
+__device__ __forceinline__ void mma_commit(uint64_t *bar)
+{
+    asm volatile("tcgen05.commit.cta_group::1.mbarrier::arrive::one.shared::cluster.b64 [%0];" ::"r"(smem_u32(bar))
+                 : "memory");
+}
+
+__device__ __forceinline__ void tmem_ld32(uint32_t taddr, float (&v)[32])
+{
+    uint32_t r[32];
+    asm volatile(
+        "tcgen05.ld.sync.aligned.32x32b.x32.b32 {%0,%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,"
+        "%16,%17,%18,%19,%20,%21,%22,%23,%24,%25,%26,%27,%28,%29,%30,%31}, [%32];"
+        : "=r"(r[0]), "=r"(r[1]), "=r"(r[2]), "=r"(r[3]), "=r"(r[4]), "=r"(r[5]), "=r"(r[6]), "=r"(r[7]),
+          "=r"(r[8]), "=r"(r[9]), "=r"(r[10]), "=r"(r[11]), "=r"(r[12]), "=r"(r[13]), "=r"(r[14]), "=r"(r[15]),
+          "=r"(r[16]), "=r"(r[17]), "=r"(r[18]), "=r"(r[19]), "=r"(r[20]), "=r"(r[21]), "=r"(r[22]), "=r"(r[23]),
+          "=r"(r[24]), "=r"(r[25]), "=r"(r[26]), "=r"(r[27]), "=r"(r[28]), "=r"(r[29]), "=r"(r[30]), "=r"(r[31])
+        : "r"(taddr));
+    asm volatile("tcgen05.wait::ld.sync.aligned;" ::: "memory");
+#pragma unroll
+    for (int i = 0; i < 32; i++) v[i] = __uint_as_float(r[i]);
+}
+
+// byte offset of element (row, k) in a K-major SW128 tile (rows of 32 fp32 = 128 B)
+__device__ __forceinline__ uint32_t kmaj_off(int row, int kchunk)
+{
+    return (uint32_t)((row >> 3) * 1024 + (row & 7) * 128 + ((kchunk ^ (row & 7)) << 4));
+}
+// byte offset of the 16-byte chunk holding (k, n..n+3) in an MN-major SW128 tile:
+// n-atoms of 32 elements at stride LBO = 4096 B (BK/8 k-groups of 1024 B each)
+__device__ __forceinline__ uint32_t mnmaj_off(int k, int nchunk)
+{
+    return (uint32_t)((nchunk >> 3) * 4096 + (k >> 3) * 1024 + (k & 7) * 128 + (((nchunk & 7) ^ (k & 7)) << 4));
+}
+
+template <int BN>
+struct Smem {
+    static constexpr int A_BYTES = BM * BK * 4;   // 16 KB
+    static constexpr int B_BYTES = BN * BK * 4;
+    static constexpr int STAGE = 2 * A_BYTES + 2 * B_BYTES;
+    static constexpr int TOTAL = STAGES * STAGE + 1024 /*align*/ + 256 /*barriers*/;
+};
+
+template <int BN, bool NT, bool NEG, bool LOWER, bool B_MN>
+__global__ void __launch_bounds__(NTHREADS, 1)
+tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const float *__restrict__ B, int ldb,
+               float *__restrict__ C, int ldc)
+{
+    using S = Smem<BN>;
+    extern __shared__ uint8_t smem_raw[];
+    uint8_t *smem = (uint8_t *)(((uintptr_t)smem_raw + 1023) & ~(uintptr_t)1023);
+    uint64_t *full = (uint64_t *)(smem + STAGES * S::STAGE);
+    uint64_t *empty = full + STAGES;
+    uint64_t *acc_full = empty + STAGES;
+    uint32_t *tmem_slot = (uint32_t *)(acc_full + 1);
+
+    const int m0 = blockIdx.y * BM, n0 = blockIdx.x * BN;
+    if (LOWER && n0 >= m0 + BM) return;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int nk = K / BK;
+
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < STAGES; s++) {
+            mbar_init(&full[s], NPROD);
+            mbar_init(&empty[s], 1);
+        }
+        mbar_init(acc_full, 1);
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    if (warp == 4) {
+        asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(tmem_slot)),
+                     "r"((uint32_t)BN));
+        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
+    }
+    tc_fence_before();
+    __syncthreads();
+    tc_fence_after();
+    const uint32_t tmem = *tmem_slot;
+
+    if (warp < 4) {
+        // ------------------------------------------------------------ producers
+        const int t = threadIdx.x;
+        constexpr int APER = BM * BK / 4 / NPROD;  // float4 per thread (8)
+        constexpr int BPER = BN * BK / 4 / NPROD;
+        float4 ra[APER], rb[BPER];
+        auto load = [&](int kb) {
+            const int k0 = kb * BK;
+#pragma unroll
+            for (int p = 0; p < APER; p++) {
+                const int f = t + p * NPROD, row = f >> 3, c = f & 7;
+                ra[p] = (m0 + row < M) ? __ldg(reinterpret_cast<const float4 *>(A + (int64_t)(m0 + row) * lda + k0 + 4 * c))
+                                       : make_float4(0.f, 0.f, 0.f, 0.f);
+            }
+#pragma unroll
+            for (int p = 0; p < BPER; p++) {
+                const int f = t + p * NPROD;
+                if (NT) {
+                    const int row = f >> 3, c = f & 7;
+                    rb[p] = (n0 + row < N) ? __ldg(reinterpret_cast<const float4 *>(B + (int64_t)(n0 + row) * ldb + k0 + 4 * c))
+                                           : make_float4(0.f, 0.f, 0.f, 0.f);
+                } else {
+                    const int kr = f / (BN / 4), nc = f % (BN / 4);
+                    rb[p] = (n0 + 4 * nc < N) ? __ldg(reinterpret_cast<const float4 *>(B + (int64_t)(k0 + kr) * ldb + n0 + 4 * nc))
+                                              : make_float4(0.f, 0.f, 0.f, 0.f);
+                }
+            }
+        };
+        auto split_store = [&](uint8_t *dst_big, uint8_t *dst_small, uint32_t off, float4 v) {
+            float4 b, s;
+            b.x = to_tf32(v.x); b.y = to_tf32(v.y); b.z = to_tf32(v.z); b.w = to_tf32(v.w);
+            s.x = v.x - b.x; s.y = v.y - b.y; s.z = v.z - b.z; s.w = v.w - b.w;
+            *reinterpret_cast<float4 *>(dst_big + off) = b;
+            *reinterpret_cast<float4 *>(dst_small + off) = s;
+        };
+        load(0);
+        for (int kb = 0; kb < nk; kb++) {
+            const int s = kb % STAGES;
+            if (kb >= STAGES) mbar_wait(&empty[s], ((kb / STAGES) - 1) & 1);
+            uint8_t *st = smem + s * S::STAGE;
+            uint8_t *a_big = st, *a_small = st + S::A_BYTES;
+            uint8_t *b_big = st + 2 * S::A_BYTES, *b_small = b_big + S::B_BYTES;
+#pragma unroll
+            for (int p = 0; p < APER; p++) {
+                const int f = t + p * NPROD, row = f >> 3, c = f & 7;
+                split_store(a_big, a_small, kmaj_off(row, c), ra[p]);
+            }
+#pragma unroll
+            for (int p = 0; p < BPER; p++) {
+                const int f = t + p * NPROD;
+                if (NT) {
+                    const int row = f >> 3, c = f & 7;
+                    split_store(b_big, b_small, kmaj_off(row, c), rb[p]);
+                } else if (B_MN) {
+                    const int kr = f / (BN / 4), nc = f % (BN / 4);
+                    split_store(b_big, b_small, mnmaj_off(kr, nc), rb[p]);
+                } else {
+                    // transpose into K-major: element (n, k) for n = 4nc..4nc+3
+                    const int kr = f / (BN / 4), nc = f % (BN / 4);
+                    const float e[4] = {rb[p].x, rb[p].y, rb[p].z, rb[p].w};
+#pragma unroll
+                    for (int q = 0; q < 4; q++) {
+                        const int n = 4 * nc + q;
+                        const uint32_t off = kmaj_off(n, kr >> 2) + (kr & 3) * 4;
+                        const float bb = to_tf32(e[q]);
+                        *reinterpret_cast<float *>(b_big + off) = bb;
+                        *reinterpret_cast<float *>(b_small + off) = e[q] - bb;
+                    }
+                }
+            }
+            fence_proxy_async();
+            mbar_arrive(&full[s]);
+            if (kb + 1 < nk) load(kb + 1);
+        }
+
+        // ------------------------------------------------------------ epilogue
+        mbar_wait(acc_full, 0);
+        tc_fence_after();
+        const int row = m0 + warp * 32 + lane;
+#pragma unroll 1
+        for (int c = 0; c < BN / 32; c++) {
+            float v[32];
+            tmem_ld32(tmem + ((uint32_t)(warp * 32) << 16) + (uint32_t)(c * 32), v);
+            if (row < M) {
+                float *crow = C + (int64_t)row * ldc + n0 + c * 32;
+#pragma unroll
+                for (int q = 0; q < 8; q++) {
+                    const int col = n0 + c * 32 + 4 * q;
+                    if (col >= N) break;
+                    float4 o = *reinterpret_cast<float4 *>(crow + 4 * q);
+                    if (LOWER && col + 3 > row) {
+                        if (col + 0 <= row) o.x += v[4 * q + 0];
+                        if (col + 1 <= row) o.y += v[4 * q + 1];
+                        if (col + 2 <= row) o.z += v[4 * q + 2];
+                        if (col + 3 <= row) o.w += v[4 * q + 3];
+                    } else {
+                        o.x += v[4 * q + 0]; o.y += v[4 * q + 1]; o.z += v[4 * q + 2]; o.w += v[4 * q + 3];
+                    }
+                    *reinterpret_cast<float4 *>(crow + 4 * q) = o;
+                }
+            }
+        }
+    } else {
+        // ------------------------------------------------------------ MMA issuer
+        constexpr uint32_t idesc = make_idesc(BM, BN, NEG, !NT && B_MN);
+        for (int kb = 0; kb < nk; kb++) {
+            const int s = kb % STAGES;
+            mbar_wait(&full[s], (kb / STAGES) & 1);
+            tc_fence_after();
+            if (lane == 0) {
+                uint8_t *st = smem + s * S::STAGE;
+                const uint32_t a_big = smem_u32(st), a_small = a_big + S::A_BYTES;
+                const uint32_t b_big = a_big + 2 * S::A_BYTES, b_small = b_big + S::B_BYTES;
+                const bool bmn = !NT && B_MN;
+#pragma unroll
+                for (int kk = 0; kk < BK / 8; kk++) {
+                    // K-major: advance 32 B inside the 128 B swizzled row; MN-major: next k-group
+                    const uint32_t ao = kk * 32, bo = bmn ? kk * 1024 : kk * 32;
+                    const uint32_t lbo = bmn ? 4096 : 16, sbo = 1024;
+                    const uint64_t dAb = make_desc(a_big + ao, 16, 1024), dAs = make_desc(a_small + ao, 16, 1024);
+                    const uint64_t dBb = make_desc(b_big + bo, lbo, sbo), dBs = make_desc(b_small + bo, lbo, sbo);
+                    const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
+                    mma_tf32(tmem, dAb, dBb, idesc, first);
+                    mma_tf32(tmem, dAb, dBs, idesc, 1u);
+                    mma_tf32(tmem, dAs, dBb, idesc, 1u);
+                }
+                mma_commit(&empty[s]);
+                if (kb == nk - 1) mma_commit(acc_full);
+            }
+            __syncwarp();
+        }
+    }
+
+    tc_fence_before();
+    __syncthreads();
+    if (warp == 4) {
+        tc_fence_after();
+        asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)BN));
+    }
+}
+
+template <bool NT, bool NEG, bool LOWER, bool B_MN = true>
+inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B, int ldb, float *C, int ldc,
+                   cudaStream_t s)
+{
+    constexpr int BN = 128;
+    if (M <= 0 || N <= 0) return 0;
+    if (K % BK) return -1;
+    auto kern = tc_gemm_kernel<BN, NT, NEG, LOWER, B_MN>;
+    constexpr int smem = Smem<BN>::TOTAL;
+    static bool attr[64] = {};
+    int dev = 0;
+    cudaGetDevice(&dev);
+    if (!attr[dev & 63]) {
+        cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+        attr[dev & 63] = true;
+    }
+    dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
+    kern<<<grid, NTHREADS, smem, s>>>(M, N, K, A, lda, B, ldb, C, ldc);
+    return 0;
+}
+
+}  // namespace tc
+
+// tc_3xtf32 versions of the five task types: the O(b^3) work on tcgen05; potrf / trsm
+// keep their small triangular panels on SIMT (simt_chol.cuh).
+inline bool tc_available(int type) { return type >= 0 && type < 5; }
+
+inline int run_tc(int type, int b, void *const *p, int *info, cudaStream_t s)
+{
+    constexpr int NBP = 64;
+    switch (type) {
+    case 0:  // MATMUL C += A B
+        return tc::tc_gemm<false, false, false>(b, b, b, (const float *)p[0], b, (const float *)p[1], b, (float *)p[2], b, s);
+    case 4:  // GEMM_NT C -= A B^T
+        return tc::tc_gemm<true, true, false>(b, b, b, (const float *)p[0], b, (const float *)p[1], b, (float *)p[2], b, s);
+    case 3:  // SYRK C -= A A^T lower
+        return tc::tc_gemm<true, true, true>(b, b, b, (const float *)p[0], b, (const float *)p[0], b, (float *)p[1], b, s);
+    case 2: {  // TRSM
+        const float *L = (const float *)p[0];
+        float *X = (float *)p[1];
+        for (int j0 = 0; j0 < b; j0 += NBP) {
+            trsm_panel<float, float, NBP>(L + (int64_t)j0 * b + j0, b, X + j0, b, b, s);
+            const int rest = b - j0 - NBP;
+            if (rest > 0)
+                tc::tc_gemm<true, true, false>(b, rest, NBP, X + j0, b, L + (int64_t)(j0 + NBP) * b + j0, b, X + j0 + NBP, b, s);
+        }
+        return 0;
+    }
+    case 1: {  // POTRF
+        float *A = (float *)p[0];
+        for (int k0 = 0; k0 < b; k0 += NBP) {
+            potrf_diag<float, float, NBP>(A + (int64_t)k0 * b + k0, b, k0, info, s);
+            const int rest = b - k0 - NBP;
+            if (rest > 0) {
+                trsm_panel<float, float, NBP>(A + (int64_t)k0 * b + k0, b, A + (int64_t)(k0 + NBP) * b + k0, b, rest, s);
+                float *P = A + (int64_t)(k0 + NBP) * b + k0;
+                tc::tc_gemm<true, true, true>(rest, rest, NBP, P, b, P, b, A + (int64_t)(k0 + NBP) * b + k0 + NBP, b, s);
+            }
+        }
+        return 0;
+    }
+    }
+    return -1;
+}
+
+}  // namespace vsk

@@ -1,0 +1,228 @@
+"""C ABI on CPU: symbol exports, and the C++ scheduler/DAG (VS_EXEC_SIM) against the
+independent Python reference model (O3) — decision logs must be identical (R22, P8)."""
+import os
+import re
+
+import pytest
+
+import paper_conf_ipps_planasbal13_b200 as vs
+from oracle.sched_model import SchedModel, submit_cholesky, submit_matmul
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+ALL = 0xFFFF
+
+
+def test_library_exports_every_header_symbol():
+    L = vs.lib()
+    hdr = open(os.path.join(ROOT, "include", "vsched.h")).read()
+    names = set(re.findall(r"^(?:int|void|uint64_t|const char \*)\s*(vs_[a-z_0-9]+)\(", hdr, re.M))
+    assert len(names) >= 25
+    for n in sorted(names):
+        assert hasattr(L, n), n
+    assert set(vs.EXPORTED) == names
+    assert "sm_100a" in vs.vs_build_info()
+
+
+def _sim(n_gpus=1, slots=4, lam=3, learning=vs.VS_LEARN_HOLD):
+    return vs.Runtime(vs.vs_config_default(exec=vs.VS_EXEC_SIM, n_gpus=n_gpus, slots_per_gpu=slots, lam=lam,
+                                           learning=learning))
+
+
+def _fake_ptr(i, nbytes):
+    return 0x10000000 + i * ((nbytes + 4095) // 4096 * 4096)
+
+
+def _pair_matmul(nt, b, lam, slots, durations, n_gpus=1):
+    """Build the same matmul workload in the C++ runtime and in the Python model."""
+    rt = _sim(n_gpus, slots, lam)
+    t = rt.vs_type_create("MATMUL", [vs.VS_IN, vs.VS_IN, vs.VS_INOUT])
+    for v in range(len(durations)):
+        rt.vs_version_add(t, "v%d" % v, ALL)
+    nbytes = b * b * 4
+    ids = [rt.vs_data_register(_fake_ptr(i, nbytes), 0, nbytes) for i in range(3 * nt * nt)]
+    A, B, C = ids[:nt * nt], ids[nt * nt:2 * nt * nt], ids[2 * nt * nt:]
+    rt.vs_app_matmul(t, nt, nt, nt, A, B, C)
+    for v, d in enumerate(durations):
+        rt.vs_replay_set(t, 3 * nbytes, v, d)
+    m = SchedModel(n_gpus, slots, lam)
+    mt = m.add_type("MATMUL", [("v%d" % v, ALL) for v in range(len(durations))])
+    mids = [m.add_data(nbytes) for _ in range(3 * nt * nt)]
+    submit_matmul(m, mt, nt, nt, nt, mids[:nt * nt], mids[nt * nt:2 * nt * nt], mids[2 * nt * nt:])
+    return rt, m
+
+
+@pytest.mark.parametrize("lam,slots", [(1, 1), (3, 4), (5, 2)])
+def test_matmul_sim_matches_reference_model(lam, slots):
+    durs = [7000, 3000]
+    rt, m = _pair_matmul(4, 256, lam, slots, durs)
+    rt.vs_wait_all()
+    ref = m.simulate(lambda ty, nb, v: durs[v])
+    got = rt.vs_decision_log()
+    assert [r[:4] for r in got] == [r[:4] for r in ref]
+    assert [(r[4], r[5]) for r in got] == [(r[4], r[5]) for r in ref]
+    assert rt.vs_decision_log_hash() == SchedModel.log_hash(ref)
+    st = rt.vs_stats()
+    assert st.tasks_completed == 64 and st.decisions == 64
+    g = rt.vs_group_stats()[0]
+    assert g["bytes"] == 786432 and g["first_reliable"] == 2 * lam + 1
+    assert g["n"] == [sum(1 for r in got if r[1] == v) for v in range(2)]
+
+
+def _pair_cholesky(nt, b, lam, slots, nv, dur, n_gpus=1):
+    rt = _sim(n_gpus, slots, lam)
+    names = ("POTRF", "TRSM", "SYRK", "GEMM_NT")
+    modes = ([vs.VS_INOUT], [vs.VS_IN, vs.VS_INOUT], [vs.VS_IN, vs.VS_INOUT], [vs.VS_IN, vs.VS_IN, vs.VS_INOUT])
+    tys = []
+    for n, md in zip(names, modes):
+        t = rt.vs_type_create(n, md)
+        for v in range(nv):
+            rt.vs_version_add(t, "v%d" % v, ALL)
+        tys.append(t)
+    nbytes = b * b * 4
+    A = {}
+    k = 0
+    for i in range(nt):
+        for j in range(i + 1):
+            A[i * nt + j] = rt.vs_data_register(_fake_ptr(k, nbytes), 0, nbytes)
+            k += 1
+    # vs_app_cholesky takes the built-in type order [MATMUL, POTRF, TRSM, SYRK, GEMM_NT]
+    rt.vs_app_cholesky([-1, tys[0], tys[1], tys[2], tys[3]], nt, A)
+    sizes = {0: nbytes, 1: 2 * nbytes, 2: 2 * nbytes, 3: 3 * nbytes}
+    for ti, t in enumerate(tys):
+        for v in range(nv):
+            rt.vs_replay_set(t, sizes[ti], v, dur(ti, sizes[ti], v))
+    m = SchedModel(n_gpus, slots, lam)
+    mt = tuple(m.add_type(n, [("v%d" % v, ALL) for v in range(nv)]) for n in names)
+    mA = {}
+    for i in range(nt):
+        for j in range(i + 1):
+            mA[i * nt + j] = m.add_data(nbytes)
+    submit_cholesky(m, mt, nt, mA)
+    return rt, m
+
+
+@pytest.mark.parametrize("nt,lam,slots,n_gpus", [(8, 3, 4, 1), (6, 1, 1, 1), (8, 2, 2, 4), (12, 3, 4, 2)])
+def test_cholesky_sim_matches_reference_model(nt, lam, slots, n_gpus):
+    dur = lambda ti, nb, v: [500, 900, 700][v] * (ti + 1) + 13 * v + ti   # noqa: E731
+    rt, m = _pair_cholesky(nt, 512, lam, slots, 3, dur, n_gpus)
+    rt.vs_wait_all()
+    ref = m.simulate(dur)
+    got = rt.vs_decision_log()
+    assert len(got) == len(ref) == nt * (nt + 1) * (nt + 2) // 6
+    assert [r[:4] for r in got] == [r[:4] for r in ref]
+    assert rt.vs_decision_log_hash() == SchedModel.log_hash(ref)
+
+
+def test_replay_bit_exact_twice():
+    dur = lambda ti, nb, v: [500, 900, 700][v] + 7 * ti   # noqa: E731
+    h = []
+    for _ in range(2):
+        rt, _m = _pair_cholesky(8, 512, 3, 4, 3, dur)
+        rt.vs_wait_all()
+        h.append(rt.vs_decision_log_hash())
+    assert h[0] == h[1]
+
+
+def test_cfg2_potrf_never_reliable_through_abi():
+    dur = lambda ti, nb, v: [500, 900, 700][v] * (ti + 1)   # noqa: E731
+    rt, _ = _pair_cholesky(8, 512, 3, 4, 3, dur)
+    rt.vs_wait_all()
+    gs = {g["type_name"]: g for g in rt.vs_group_stats()}
+    assert not gs["POTRF"]["reliable"] and sum(gs["POTRF"]["n"]) == 8
+    assert gs["GEMM_NT"]["reliable"] and gs["GEMM_NT"]["first_reliable"] == 10
+
+
+def test_table_i_and_new_group(tmp_path):
+    MB = 1 << 20
+    p = tmp_path / "table.txt"
+    p.write_text("task1 %d task1-v1 30000000 200\ntask1 %d task1-v2 18000000 350\ntask1 %d task1-v3 25000000 230\n"
+                 "task1 %d task1-v1 45000000 80\ntask1 %d task1-v2 25000000 300\ntask1 %d task1-v3 40000000 120\n"
+                 "task2 %d task2-v1 15000000 40\ntask2 %d task2-v2 20000000 3\n"
+                 % (2 * MB, 2 * MB, 2 * MB, 3 * MB, 3 * MB, 3 * MB, 5 * MB, 5 * MB))
+    for lam, expect_v2 in ((3, 0), (4, 1)):
+        rt = _sim(2, 1, lam)
+        t1 = rt.vs_type_create("task1", [vs.VS_INOUT])
+        for v in ("task1-v1", "task1-v2", "task1-v3"):
+            rt.vs_version_add(t1, v, ALL)
+        t2 = rt.vs_type_create("task2", [vs.VS_INOUT])
+        for v in ("task2-v1", "task2-v2"):
+            rt.vs_version_add(t2, v, ALL)
+        rt.vs_table_load(str(p))
+        d2 = rt.vs_data_register(_fake_ptr(0, 2 * MB), 0, 2 * MB)
+        d3 = rt.vs_data_register(_fake_ptr(1, 4 * MB), 0, 3 * MB)
+        d5 = rt.vs_data_register(_fake_ptr(3, 6 * MB), 0, 5 * MB)
+        d4 = rt.vs_data_register(_fake_ptr(5, 6 * MB), 0, 4 * MB)
+        for t, d in ((t1, d2), (t1, d3), (t2, d5), (t1, d4)):
+            rt.vs_submit(t, [d])
+        for t, nb, nv in ((t1, 2 * MB, 3), (t1, 3 * MB, 3), (t2, 5 * MB, 2), (t1, 4 * MB, 3)):
+            for v in range(nv):
+                rt.vs_replay_set(t, nb, v, 1000)
+        rt.vs_wait_all()
+        log = rt.vs_decision_log()
+        assert log[0][1] == 1 and log[0][6] == 1          # task1 @2MB -> v2, reliable
+        assert log[1][1] == 1 and log[1][6] == 1          # task1 @3MB -> v2
+        assert log[2][1] == expect_v2                      # task2 @5MB: v1 (lam 3) / v2 learning (lam 4)
+        assert log[2][6] == (1 if lam == 3 else 0)
+        assert log[3][6] == 0 and log[3][1] == 0           # new size 4MB -> learning, RR from v1
+        out = tmp_path / ("dump%d.txt" % lam)
+        rt.vs_table_dump(str(out))
+        assert "task1 %d task1-v1 45000000 80" % (3 * MB) in out.read_text()   # untouched group entry
+
+
+def test_fig5_earliest_executor_masks():
+    # Fig 5: version "fast" runs only on gpu 3 (worker 3), "slow" only on gpu 2.
+    rt = _sim(4, 1, 1)
+    t = rt.vs_type_create("task", [vs.VS_INOUT])
+    rt.vs_version_add(t, "fast", 1 << 3)
+    rt.vs_version_add(t, "slow", 1 << 2)
+    ds = [rt.vs_data_register(_fake_ptr(i, 64), 0, 64) for i in range(8)]
+    for d in ds:
+        rt.vs_submit(t, [d])
+    rt.vs_replay_set(t, 64, 0, 10_000)
+    rt.vs_replay_set(t, 64, 1, 40_000)
+    rt.vs_wait_all()
+    log = rt.vs_decision_log()
+    m = SchedModel(4, 1, 1)
+    mt = m.add_type("task", [("fast", 1 << 3), ("slow", 1 << 2)])
+    for _ in range(8):
+        m.submit(mt, [(m.add_data(64), "inout")])
+    ref = m.simulate(lambda ty, nb, v: [10_000, 40_000][v])
+    assert [r[:4] for r in log] == [r[:4] for r in ref]
+    # after learning, tasks pile on worker 3 until its backlog exceeds 40 us, then worker 2 helps
+    reliable = [r for r in log if r[6] == 1]
+    assert any(r[2] == 2 for r in reliable) and any(r[2] == 3 for r in reliable)
+
+
+def test_overlap_and_errors():
+    rt = _sim()
+    a = rt.vs_data_register(0x1000, 0, 4096)
+    assert rt.vs_data_register(0x1000, 0, 4096) == a
+    with pytest.raises(vs.VSError) as e:
+        rt.vs_data_register(0x1800, 0, 4096)
+    assert e.value.code == vs.VS_E_OVERLAP
+    t = rt.vs_type_create("x", [vs.VS_INOUT])
+    with pytest.raises(vs.VSError):
+        rt.vs_submit(t, [a])        # no version
+    rt.vs_version_add(t, "v", ALL)
+    with pytest.raises(vs.VSError):
+        rt.vs_submit(t, [a, a])     # wrong arity
+    rt.vs_submit(t, [a])
+    with pytest.raises(vs.VSError) as e:
+        rt.vs_wait_all()            # no replay duration
+    assert e.value.code == vs.VS_E_STATE
+
+
+def test_rr_learning_variant_keeps_cycling():
+    rt = _sim(1, 4, 2, learning=vs.VS_LEARN_RR)
+    t = rt.vs_type_create("x", [vs.VS_INOUT])
+    rt.vs_version_add(t, "a", ALL)
+    rt.vs_version_add(t, "b", ALL)
+    ds = [rt.vs_data_register(_fake_ptr(i, 64), 0, 64) for i in range(12)]
+    for d in ds:
+        rt.vs_submit(t, [d])
+    rt.vs_replay_set(t, 64, 0, 100)
+    rt.vs_replay_set(t, 64, 1, 50)
+    rt.vs_wait_all()
+    log = rt.vs_decision_log()
+    # all 12 are ready at t=0, no time has been recorded yet: paper-literal RR alternates
+    assert [r[1] for r in log] == [0, 1] * 6
