@@ -1,0 +1,429 @@
+"""bench.py — tiled matmul + tiled Cholesky GFLOP/s under the versioning scheduler (B200).
+
+One STEP = one pass of the whole hot path over one batch of synthetic input: the tiled
+matmul of cfg3 (N=16384 fp32, 1024x1024 tiles, 4096 MATMUL tasks) and the tiled
+Cholesky of cfg4 (N=32768 SPD fp32, 1024x1024 tiles, 5984 potrf/trsm/syrk/gemm tasks),
+submitted together through the C ABI (vs_app_matmul + vs_app_cholesky) and run to
+completion by vs_wait_all: registration -> dependence analysis -> versioning decisions
+(learning, then earliest executor) -> device-enforced dependences -> sm_100a tile kernels.
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+
+value  = (2*16384^3 + 32768^3/3) flops per step x steps x ranks / max-over-ranks time.
+N > 1: one process per GPU (torchrun); each rank runs an independent instance of the
+step on its own GPU (weak scaling, no data-path collective).
+--impl reference: the CPU oracle (oracle/) timed on this host's cores on a bounded
+sample of the same workload (the tier's reference arm).
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import math
+import os
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+MM_N, MM_B = 16384, 1024
+CH_N, CH_B = 32768, 1024
+SEED_MM, SEED_CH = 3, 4
+F32_VERSIONS_MASK = 0b111     # simt_f32 | tc_3xtf32 | f64in_f32io
+MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
+CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
+
+
+def peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        d = json.load(open(p))
+        return d, "measured"
+    return {"hbm_gbs": 6650.0, "bf16_tflops": 1590.0, "bf16_tflops_sustained": 1400.0, "sm_max_mhz": 1965.0}, "fallback"
+
+
+# ----------------------------------------------------------------------------- workload
+class Workload:
+    """Device-resident (or pinned-host, for e2e) tiles of cfg3 + cfg4 and their data ids."""
+
+    def __init__(self, rt, mm_n=MM_N, mm_b=MM_B, ch_n=CH_N, ch_b=CH_B, host=False, seed_off=0, mask=F32_VERSIONS_MASK,
+                 with_mm=True, with_ch=True):
+        import torch
+        import paper_conf_ipps_planasbal13_b200 as vs
+        self.torch, self.vs, self.rt = torch, vs, rt
+        self.mm_n, self.mm_b, self.ch_n, self.ch_b, self.host = mm_n, mm_b, ch_n, ch_b, host
+        self.with_mm, self.with_ch = with_mm, with_ch
+        self.types = rt.vs_register_builtins(vs.VS_F32, mask)
+        dev = torch.device("cuda")
+        dev_i = -1 if host else 0
+        self.flops = 0.0
+        if with_mm:
+            nt = mm_n // mm_b
+            self.mm_nt = nt
+            # generated on the device by vs_gen_uniform (bit-identical to vsgen)
+            gA = torch.empty((nt, nt, mm_b, mm_b), dtype=torch.float32, device=dev)
+            gB = torch.empty_like(gA)
+            vs.vs_gen_uniform(SEED_MM + seed_off, mm_n, mm_n, vs.VS_F32, mm_b, gA.data_ptr())
+            vs.vs_gen_uniform(SEED_MM + 1000 + seed_off, mm_n, mm_n, vs.VS_F32, mm_b, gB.data_ptr())
+            if host:
+                self.A = gA.cpu().pin_memory()
+                self.B = gB.cpu().pin_memory()
+                self.C = torch.zeros_like(self.A).pin_memory()
+                del gA, gB
+            else:
+                self.A, self.B = gA, gB
+                self.C = torch.zeros_like(gA)
+            nb = mm_b * mm_b * 4
+            reg = lambda T: [rt.vs_data_register(T[i, j].data_ptr(), dev_i, nb) for i in range(nt) for j in range(nt)]  # noqa
+            self.ia, self.ib, self.ic = reg(self.A), reg(self.B), reg(self.C)
+            self.flops += MM_FLOPS(mm_n)
+        if with_ch:
+            nt = ch_n // ch_b
+            self.ch_nt = nt
+            g = torch.empty((nt, nt, ch_b, ch_b), dtype=torch.float32, device=dev)
+            vs.vs_gen_spd(SEED_CH + seed_off, ch_n, vs.VS_F32, ch_b, g.data_ptr())
+            if host:
+                self.S0 = g.cpu()
+                self.S = self.S0.clone().pin_memory()
+                del g
+            else:
+                self.S0 = g
+                self.S = g.clone()
+            nb = ch_b * ch_b * 4
+            self.iS = {i * nt + j: rt.vs_data_register(self.S[i, j].data_ptr(), dev_i, nb)
+                       for i in range(nt) for j in range(i + 1)}
+            self.flops += CH_FLOPS(ch_n)
+        torch.cuda.synchronize()
+
+    def reset(self):
+        """Restore the step's inputs (C = 0, A_chol = pristine).  Device: async on torch's
+        stream + sync; host: memcpy (outside the timed region for e2e)."""
+        if self.with_mm:
+            self.C.zero_()
+        if self.with_ch:
+            self.S.copy_(self.S0)
+        if not self.host:
+            self.torch.cuda.current_stream().synchronize()
+
+    def submit(self):
+        vs, rt = self.vs, self.rt
+        if self.with_mm:
+            nt = self.mm_nt
+            rt.vs_app_matmul(self.types[vs.VS_T_MATMUL], nt, nt, nt, self.ia, self.ib, self.ic)
+        if self.with_ch:
+            rt.vs_app_cholesky(self.types, self.ch_nt, self.iS)
+
+    def step(self):
+        self.reset()
+        self.submit()
+        self.rt.vs_wait_all()
+
+
+# ----------------------------------------------------------------------------- clocks
+class ClockSampler:
+    Q = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
+         "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+         "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index):
+        self.index = index
+        self.rows = []
+        self.proc = None
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(["nvidia-smi", "-i", str(self.index), "--query-gpu=" + self.Q,
+                                          "--format=csv,noheader,nounits", "-lms", "200"],
+                                         stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.th = threading.Thread(target=self._read, daemon=True)
+            self.th.start()
+        except Exception:
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.rows.append([x.strip() for x in line.split(",")])
+
+    def stop(self):
+        if self.proc:
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except Exception:
+                self.proc.kill()
+        rows = [r for r in self.rows if len(r) >= 9]
+        if not rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unavailable"], "samples": 0}
+        sm = sorted(float(r[1]) for r in rows if r[1].replace(".", "").isdigit())
+        mx = max(float(r[2]) for r in rows if r[2].replace(".", "").isdigit())
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for r in rows for i in range(4) if r[5 + i].lower().startswith("active")})
+        return {"sm_mhz": sm[len(sm) // 2] if sm else None, "sm_max_mhz": mx, "reasons": reasons, "samples": len(rows)}
+
+
+# ----------------------------------------------------------------------------- roofline
+def union_ns(intervals):
+    tot, cur_s, cur_e = 0, None, None
+    for s, e in sorted(intervals):
+        if cur_e is None or s > cur_e:
+            if cur_e is not None:
+                tot += cur_e - cur_s
+            cur_s, cur_e = s, e
+        else:
+            cur_e = max(cur_e, e)
+    if cur_e is not None:
+        tot += cur_e - cur_s
+    return tot
+
+
+def task_flops(type_name, b):
+    t = type_name.split(".")[0]
+    return {"MATMUL": 2.0 * b ** 3, "GEMM_NT": 2.0 * b ** 3, "SYRK": 1.0 * b ** 3, "TRSM": 1.0 * b ** 3,
+            "POTRF": b ** 3 / 3.0}[t]
+
+
+# ----------------------------------------------------------------------------- reference arm
+def cpu_sample(target_s=12.0):
+    """The oracle as it stands, on a bounded sample of the same workload:
+    matmul rows 0..R-1 of C = A*B at N=16384 (fp64, plain i,k,j loop) and the Cholesky of
+    the leading k x k block of the cfg4 SPD matrix (L[:k,:k] = chol(A[:k,:k]))."""
+    import numpy as np
+
+    import oracle
+    import vsgen
+    cores = len(os.sched_getaffinity(0))
+    os.environ.setdefault("OMP_NUM_THREADS", str(cores))
+    # calibrate rows: one row of C costs 2*N^2 flops
+    A_rows = vsgen.uniform(SEED_MM, 64, MM_N)
+    B = vsgen.uniform_idx(SEED_MM + 1000, np.arange(MM_N * MM_N, dtype=np.uint64)).reshape(MM_N, MM_N)
+    t0 = time.perf_counter()
+    oracle.matmul(A_rows[:8], B)
+    dt8 = time.perf_counter() - t0
+    rows = int(max(8, min(64, 8 * (target_s / 2) / max(dt8, 1e-3))))
+    t0 = time.perf_counter()
+    oracle.matmul(A_rows[:rows], B)
+    t_mm = time.perf_counter() - t0
+    f_mm = 2.0 * rows * MM_N * MM_N
+    k = 2048
+    # leading k x k block of the N=32768 SPD matrix (same generator, global indices)
+    r = np.arange(k, dtype=np.uint64)[:, None]
+    c = np.arange(k, dtype=np.uint64)[None, :]
+    hi, lo = np.maximum(r, c), np.minimum(r, c)
+    S = vsgen.uniform_idx(SEED_CH, hi * np.uint64(CH_N) + lo)
+    S[np.arange(k), np.arange(k)] += vsgen.spd_alpha(CH_N)
+    S = S.astype(np.float32)
+    t0 = time.perf_counter()
+    _, info = oracle.cholesky(S)
+    t_ch = time.perf_counter() - t0
+    f_ch = k ** 3 / 3.0
+    return {"t_mm": t_mm, "f_mm": f_mm, "rows": rows, "t_ch": t_ch, "f_ch": f_ch, "k": k, "cores": cores,
+            "info": info}
+
+
+def run_reference(args, rank, world):
+    if rank != 0:
+        return 0
+    samples = []
+    for i in range(args.warmup + args.steps):
+        s = cpu_sample(target_s=4.0)
+        if i >= args.warmup:
+            samples.append(s)
+    t = sum(s["t_mm"] + s["t_ch"] for s in samples)
+    f = sum(s["f_mm"] + s["f_ch"] for s in samples)
+    gf = f / t / 1e9
+    s0 = samples[0]
+    sample = ("per step: oracle fp64 matmul rows 0..%d of C=A*B at N=16384 + oracle unblocked Cholesky of the "
+              "leading %dx%d block of the cfg4 SPD matrix" % (s0["rows"] - 1, s0["k"], s0["k"]))
+    out = {"metric": "tiled matmul & Cholesky GFLOP/s", "value": round(gf, 3), "unit": "GFLOP/s", "impl": "reference",
+           "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
+           "ms_per_step": round(1e3 * t / len(samples), 2), "higher_is_better": True, "scaling": "weak",
+           "vs_baseline": None, "dtype": "f64", "data": "synthetic (vsgen counter-based generator)",
+           "config": {"workload": "cfg3+cfg4 (bounded CPU sample)", "matmul_N": MM_N, "cholesky_N": CH_N},
+           "cpu_baseline": {"value": round(gf, 3), "unit": "GFLOP/s", "cores": s0["cores"], "kind": "oracle",
+                            "sample": sample},
+           "e2e": {"value": round(gf, 3), "unit": "GFLOP/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(out))
+    return 0
+
+
+# ----------------------------------------------------------------------------- our arm
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--slots", type=int, default=int(os.environ.get("VS_SLOTS", "4")))
+    ap.add_argument("--lam", type=int, default=3)
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--small", action="store_true", help="cfg1/cfg2-sized smoke of the bench itself")
+    ap.add_argument("--only", choices=["mm", "ch", "both"], default="both")
+    ap.add_argument("--dump-log", default="")
+    args = ap.parse_args()
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if args.impl == "reference":
+        return run_reference(args, rank, world)
+
+    import torch
+    import paper_conf_ipps_planasbal13_b200 as vs
+    torch.cuda.set_device(local)
+    dist = None
+    if world > 1:
+        import torch.distributed as dist
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+
+    def barrier():
+        if dist is not None:
+            dist.barrier()
+
+    mm_n, mm_b, ch_n, ch_b = (MM_N, MM_B, CH_N, CH_B) if not args.small else (1024, 256, 4096, 512)
+    with_mm, with_ch = args.only in ("mm", "both"), args.only in ("ch", "both")
+    cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0)
+    rt = vs.Runtime(cfg)
+    wl = Workload(rt, mm_n, mm_b, ch_n, ch_b, host=False, seed_off=rank, with_mm=with_mm, with_ch=with_ch)
+
+    # warm-up (the first step includes the learning phase: "cold")
+    t0 = time.perf_counter()
+    wl.step()
+    cold_ms = (time.perf_counter() - t0) * 1e3
+    for _ in range(args.warmup - 1):
+        wl.step()
+    rt.vs_decision_log_clear()
+    st0 = rt.vs_stats()
+
+    sampler = ClockSampler(local)
+    sampler.start()
+    time.sleep(0.3)
+    barrier()
+    torch.cuda.synchronize()
+    ev0, ev1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    ev0.record()
+    for _ in range(args.steps):
+        wl.step()
+    ev1.record()
+    torch.cuda.synchronize()
+    barrier()
+    ms = ev0.elapsed_time(ev1)
+    clocks = sampler.stop()
+    if dist is not None:
+        t = torch.tensor([ms], device="cuda")
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        ms = float(t.item())
+    st1 = rt.vs_stats()
+    log = rt.vs_decision_log()
+    groups = rt.vs_group_stats()
+    ms_step = ms / args.steps
+    gflops = wl.flops * args.steps * world / (ms * 1e-3) / 1e9
+
+    # ---- roofline of the dominant kernel (the (type, version) carrying most flops in the timed steps)
+    pk, pk_kind = peaks()
+    tf32_peak = pk.get("bf16_tflops_sustained", pk["bf16_tflops"]) * 0.5   # TF32 = 1/2 BF16 (nominal ratio)
+    tnames = {g["type"]: g["type_name"] for g in groups}
+    vnames = {g["type"]: g["versions"] for g in groups}
+    tile_b = {}
+    for g in groups:
+        npar = {"MATMUL": 3, "GEMM_NT": 3, "SYRK": 2, "TRSM": 2, "POTRF": 1}[g["type_name"].split(".")[0]]
+        tile_b[g["type"]] = int(round(math.sqrt(g["bytes"] / 4 / npar)))
+    per = {}
+    for (task, v, w, td, ts, te, ph, ty) in log:
+        key = (tnames[ty], vnames[ty][v])
+        d = per.setdefault(key, {"n": 0, "flops": 0.0, "iv": [], "busy_ns": 0})
+        d["n"] += 1
+        d["flops"] += task_flops(tnames[ty], tile_b[ty])
+        d["iv"].append((ts, te))
+        d["busy_ns"] += te - ts
+    dom = max(per, key=lambda k: per[k]["flops"])
+    d = per[dom]
+    union = union_ns(d["iv"])
+    hw = 3.0 if dom[1] == "tc_3xtf32" else 1.0
+    achieved = hw * d["flops"] / (union * 1e-9) / 1e12          # TFLOP/s while that kernel class runs
+    if dom[1] == "tc_3xtf32":
+        peak, unit, bound = tf32_peak, "TFLOP/s", "tensor"
+    else:
+        peak, unit, bound = 148 * 128 * 2 * pk["sm_max_mhz"] * 1e6 / 1e12, "TFLOP/s", "alu"
+    tc_flops = sum(v["flops"] for k, v in per.items() if k[1] == "tc_3xtf32")
+    tensor_frac_step = 3.0 * tc_flops / (ms * 1e-3 / world) / 1e12 / tf32_peak if world == 1 else None
+    version_counts = {"%s/%s" % k: v["n"] for k, v in sorted(per.items())}
+    launches = st1.kernel_launches - st0.kernel_launches
+
+    # ---- e2e: same step through the C ABI with HOST (pinned) buffers, copies inside the timed region
+    e2e = None
+    if not args.no_e2e:
+        rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots))
+        wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, seed_off=rank, with_mm=with_mm, with_ch=with_ch)
+        wl2.step()     # warm-up incl. learning
+        tsum, h2d, d2h = 0.0, 0, 0
+        n_e2e = 2
+        for _ in range(n_e2e):
+            wl2.reset()
+            s0 = rt2.vs_stats()
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            wl2.submit()
+            rt2.vs_wait_all()            # includes the flush of written tiles to host (Output Tx)
+            torch.cuda.synchronize()
+            tsum += time.perf_counter() - t0
+            s1 = rt2.vs_stats()
+            h2d += s1.input_tx_bytes - s0.input_tx_bytes
+            d2h += s1.output_tx_bytes - s0.output_tx_bytes
+        e2e = {"value": round(wl2.flops * n_e2e / tsum / 1e9, 1), "unit": "GFLOP/s",
+               "h2d_bytes_per_step": int(h2d // n_e2e), "d2h_bytes_per_step": int(d2h // n_e2e)}
+        rt2.close()
+        del wl2
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu:
+        s = cpu_sample()
+        cpu = {"value": round((s["f_mm"] + s["f_ch"]) / (s["t_mm"] + s["t_ch"]) / 1e9, 3), "unit": "GFLOP/s",
+               "cores": s["cores"], "kind": "oracle",
+               "sample": "oracle fp64 matmul rows 0..%d of C=A*B at N=%d (%.1f s) + oracle unblocked Cholesky of the "
+                         "leading %dx%d block of the cfg4 SPD matrix (%.1f s)" % (
+                             s["rows"] - 1, MM_N, s["t_mm"], s["k"], s["k"], s["t_ch"])}
+
+    if rank == 0:
+        out = {
+            "metric": "tiled matmul & Cholesky GFLOP/s", "value": round(gflops, 1), "unit": "GFLOP/s",
+            "n_gpus": world, "steps": args.steps, "warmup": args.warmup, "ms_per_step": round(ms_step, 3),
+            "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f32",
+            "data": "synthetic (counter-based generator; U(-1,1) matmul operands, SPD A = S + 2.5 sqrt(N) I)",
+            "config": {"workload": ("cfg3+cfg4: tiled matmul N=%d b=%d + tiled Cholesky N=%d b=%d, fp32, versions "
+                                    "simt_f32/tc_3xtf32/f64in_f32io, lambda=%d, %d slots/GPU" % (
+                                        mm_n, mm_b, ch_n, ch_b, args.lam, args.slots)) if with_mm and with_ch else
+                       args.only,
+                       "matmul_N": mm_n if with_mm else None, "cholesky_N": ch_n if with_ch else None,
+                       "tile": mm_b, "lambda": args.lam, "slots_per_gpu": args.slots,
+                       "parallelism": "independent instance per GPU" if world > 1 else "1 GPU",
+                       "l2": "inputs larger than L2 (4 GiB + 4 GiB per GPU)", "regime": "warm (tables learned in warm-up)"},
+            "parts_gflop": {"matmul": MM_FLOPS(mm_n) / 1e9 if with_mm else 0, "cholesky": CH_FLOPS(ch_n) / 1e9 if with_ch else 0},
+            "cold_first_step_ms": round(cold_ms, 1),
+            "tensor_pipe_fraction_step": round(tensor_frac_step, 4) if tensor_frac_step is not None else None,
+            "roofline": {"bound": bound, "kernel": "%s/%s b=%d" % (dom[0], dom[1], tile_b[[t for t in tnames if tnames[t] == dom[0]][0]]),
+                         "achieved": round(achieved, 2), "peak": round(peak, 1), "unit": unit,
+                         "frac": round(achieved / peak, 4), "traffic": None,
+                         "peak_source": "%s bf16_tflops_sustained x 0.5 (TF32/BF16 nominal ratio)" % pk_kind
+                         if bound == "tensor" else "148 SM x 128 FMA x 2 x sm_max_mhz",
+                         "how": "hardware MMA flops (3x algorithmic) of all launches of this kernel class in the "
+                                "timed steps / union of their CUDA-event intervals on the worker streams"},
+            "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
+            "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
+            "version_counts": version_counts,
+            "host_us_per_task": {"decide": round((st1.host_ns_decide - st0.host_ns_decide) / 1e3 / max(1, len(log)), 3),
+                                 "issue": round((st1.host_ns_issue - st0.host_ns_issue) / 1e3 / max(1, len(log)), 3)},
+        }
+        print(json.dumps(out))
+        if args.dump_log:
+            json.dump({"log": log, "groups": groups}, open(args.dump_log, "w"))
+    rt.close()
+    if dist is not None:
+        dist.destroy_process_group()
+    return 0
+
+
+if __name__ == "__main__":
+    sys.exit(main() or 0)

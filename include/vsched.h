@@ -186,6 +186,7 @@ typedef struct {
     int64_t host_ns_decide;   /* host time spent in decisions (scheduler overhead) */
     int64_t host_ns_issue;    /* host time spent issuing GPU work */
     int64_t virtual_now_ns;   /* DES clock */
+    int64_t kernel_launches;  /* process-wide count of libvsched kernel launches */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 
@@ -211,9 +212,11 @@ const char *vs_version_name(vs_rt rt, vs_type_id t, vs_version_id v);
 typedef struct {
     vs_task_id task;
     int32_t version, worker;   /* worker = gpu * slots_per_gpu + slot */
-    int32_t phase, pad;        /* 0 learning, 1 reliable */
+    int32_t phase;             /* 0 learning, 1 reliable */
+    vs_type_id type;           /* task type */
     int64_t t_decide_ns;       /* virtual (run-ahead / sim) or host clock (ready) */
-    int64_t t_start_ns, t_end_ns; /* sim: virtual; gpu: measured start/end (0 if unknown) */
+    int64_t t_start_ns, t_end_ns; /* sim: virtual clock; gpu: GPU timeline of the version's
+                                     start/end events (ns since runtime creation) */
 } vs_decision_t;
 /* Copy up to cap records (from the beginning) into out; *n = total records. */
 int vs_decision_log(vs_rt rt, vs_decision_t *out, int64_t cap, int64_t *n);

@@ -45,7 +45,8 @@ class vs_config(Structure):
 class vs_stats_t(Structure):
     _fields_ = [(n, c_int64) for n in (
         "tasks_submitted", "tasks_completed", "decisions", "input_tx_bytes", "output_tx_bytes", "device_tx_bytes",
-        "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns")]
+        "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns",
+        "kernel_launches")]
 
 
 class vs_group_stat_t(Structure):
@@ -56,7 +57,7 @@ class vs_group_stat_t(Structure):
 
 
 class vs_decision_t(Structure):
-    _fields_ = [("task", c_int64), ("version", c_int32), ("worker", c_int32), ("phase", c_int32), ("pad", c_int32),
+    _fields_ = [("task", c_int64), ("version", c_int32), ("worker", c_int32), ("phase", c_int32), ("type", c_int32),
                 ("t_decide_ns", c_int64), ("t_start_ns", c_int64), ("t_end_ns", c_int64)]
 
 
@@ -266,7 +267,7 @@ class Runtime:
         lib().vs_decision_log(self.h, None, 0, ctypes.byref(n))
         buf = (vs_decision_t * max(1, n.value))()
         lib().vs_decision_log(self.h, buf, n.value, ctypes.byref(n))
-        return [(r.task, r.version, r.worker, r.t_decide_ns, r.t_start_ns, r.t_end_ns, r.phase)
+        return [(r.task, r.version, r.worker, r.t_decide_ns, r.t_start_ns, r.t_end_ns, r.phase, r.type)
                 for r in buf[:n.value]]
 
     def vs_decision_log_hash(self) -> int:

@@ -64,6 +64,7 @@ __global__ void gen_spd_kernel(uint64_t seed, int64_t n, int tile_b, double alph
 int gen_uniform(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b, void *out, cudaStream_t s)
 {
     const int grid = 148 * 16;
+    count_launch();
     if (dtype == 0) gen_uniform_kernel<float><<<grid, 256, 0, s>>>(seed, rows, cols, tile_b, (float *)out);
     else if (dtype == 1) gen_uniform_kernel<double><<<grid, 256, 0, s>>>(seed, rows, cols, tile_b, (double *)out);
     else return -1;
@@ -74,6 +75,7 @@ int gen_spd(uint64_t seed, int64_t n, int dtype, int tile_b, void *out, cudaStre
 {
     const double alpha = n >= 256 ? 2.5 * std::sqrt((double)n) : (double)n;  // reading R8
     const int grid = 148 * 16;
+    count_launch();
     if (dtype == 0) gen_spd_kernel<float><<<grid, 256, 0, s>>>(seed, n, tile_b, alpha, (float *)out);
     else if (dtype == 1) gen_spd_kernel<double><<<grid, 256, 0, s>>>(seed, n, tile_b, alpha, (double *)out);
     else return -1;

@@ -4,7 +4,17 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 
+#include <atomic>
+
 namespace vsk {
+
+// Process-wide count of kernels launched by libvsched (reported as gpu_launches).
+inline std::atomic<long long> &launch_counter()
+{
+    static std::atomic<long long> c{0};
+    return c;
+}
+inline void count_launch() { launch_counter().fetch_add(1, std::memory_order_relaxed); }
 
 // Task types / versions use the VS_T_* / VS_V_* numbering of vsched.h.
 // Returns 0 on success, -1 for an unsupported (type, version, b).

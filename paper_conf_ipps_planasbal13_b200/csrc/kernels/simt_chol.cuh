@@ -13,6 +13,8 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 
+#include "kernels.hpp"
+
 namespace vsk {
 
 // Unblocked right-looking Cholesky of an NB x NB diagonal block at A (leading dim lda),
@@ -92,6 +94,7 @@ __global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, T
 template <typename Tin, typename Tacc, int NB>
 inline void potrf_diag(Tin *A, int lda, int k_base, int *info, cudaStream_t s)
 {
+    count_launch();
     potrf_diag_kernel<Tin, Tacc, NB><<<1, 256, 0, s>>>(A, lda, k_base, info);
 }
 
@@ -99,6 +102,7 @@ template <typename Tin, typename Tacc, int NB>
 inline void trsm_panel(const Tin *L, int ldl, Tin *X, int ldx, int rows, cudaStream_t s)
 {
     if (rows <= 0) return;
+    count_launch();
     trsm_panel_kernel<Tin, Tacc, NB><<<(rows + 63) / 64, 64, 0, s>>>(L, ldl, X, ldx, rows);
 }
 

@@ -19,6 +19,8 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 
+#include "kernels.hpp"
+
 namespace vsk {
 
 template <typename T> struct Vec16;
@@ -147,6 +149,7 @@ inline void simt_gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, 
     constexpr bool WIDE = sizeof(Tacc) == 4;           // fp32 math: 128x128 tiles, 8x8 per thread
     constexpr int BM = WIDE ? 128 : 64, BN = WIDE ? 128 : 64, BK = 16, TM = WIDE ? 8 : 4, TN = WIDE ? 8 : 4;
     dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
+    count_launch();
     simt_gemm_kernel<Tin, Tacc, BM, BN, BK, TM, TN, NT, NEG, LOWER>
         <<<grid, (BM / TM) * (BN / TN), 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc);
 }

@@ -23,6 +23,8 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 
+#include "kernels.hpp"
+
 namespace vsk {
 namespace tc {
 
@@ -328,6 +330,7 @@ inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B,
         attr[dev & 63] = true;
     }
     dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
+    count_launch();
     kern<<<grid, NTHREADS, smem, s>>>(M, N, K, A, lda, B, ldb, C, ldc);
     return 0;
 }

@@ -1,0 +1,173 @@
+"""End-to-end GPU runs through the C ABI runtime (versioning scheduler + device-enforced
+dependences + tile kernels) on the BASELINE.json configs, against the CPU oracle."""
+import numpy as np
+import pytest
+
+import oracle
+import paper_conf_ipps_planasbal13_b200 as vs
+import vsgen
+
+pytestmark = pytest.mark.gpu
+
+F32_MASK = (1 << vs.VS_V_SIMT_F32) | (1 << vs.VS_V_TC_3XTF32) | (1 << vs.VS_V_F64IN_F32IO)
+
+
+def _torch():
+    import torch
+    return torch
+
+
+def _tiles_dev(a, b):
+    torch = _torch()
+    t = vsgen.to_tiles(a, b)
+    return torch.from_numpy(t).cuda()
+
+
+def _register_tiles(rt, T, device=0):
+    """T: tensor (mt, nt, b, b) on cuda (device=0) or pinned host (device=-1)."""
+    mt, nt, b, _ = T.shape
+    nbytes = b * b * T.element_size()
+    return [rt.vs_data_register(T[i, j].data_ptr(), device, nbytes) for i in range(mt) for j in range(nt)]
+
+
+def _matmul(rt, N, b, dtype=vs.VS_F32, mask=F32_MASK, seed=1, C0=None, host=False):
+    torch = _torch()
+    nt = N // b
+    types = rt.vs_register_builtins(dtype, mask)
+    npdt = np.float32 if dtype == vs.VS_F32 else np.float64
+    A = vsgen.uniform(seed, N, N, npdt)
+    B = vsgen.uniform(seed + 1000, N, N, npdt)
+    C = np.zeros((N, N), npdt) if C0 is None else C0
+    if host:
+        tA, tB, tC = (torch.from_numpy(vsgen.to_tiles(x, b)).pin_memory() for x in (A, B, C))
+        dev = -1
+    else:
+        tA, tB, tC = (_tiles_dev(x, b) for x in (A, B, C))
+        dev = 0
+    ia, ib, ic = (_register_tiles(rt, t, dev) for t in (tA, tB, tC))
+    rt.vs_app_matmul(types[vs.VS_T_MATMUL], nt, nt, nt, ia, ib, ic)
+    rt.vs_wait_all()
+    torch.cuda.synchronize()
+    return A, B, C, vsgen.from_tiles(tC.cpu().numpy())
+
+
+def test_cfg1_matmul_versioning(gpu):
+    # cfg1: matmul N=1024 fp32, 256x256 tiles, 2 versions, lambda = 3
+    rt = vs.Runtime(lam=3)
+    mask = (1 << vs.VS_V_SIMT_F32) | (1 << vs.VS_V_TC_3XTF32)
+    C0 = vsgen.uniform(2001, 1024, 1024)
+    A, B, C0, C = _matmul(rt, 1024, 256, mask=mask, C0=C0)
+    ref = oracle.matmul(A, B, C0)
+    assert oracle.relF(C, ref) <= 1e-5
+    g = rt.vs_group_stats()[0]
+    assert g["bytes"] == 786432 and sum(g["n"]) == 64
+    assert all(n >= 3 for n in g["n"])                  # each version ran >= lambda times
+    assert g["reliable"] and g["first_reliable"] == 7   # V*lambda + 1 with hold
+    st = rt.vs_stats()
+    assert st.tasks_completed == 64 and st.input_tx_bytes == 0
+    rt.close()
+
+
+def test_matmul_host_data_copy_deps(gpu):
+    # e2e path: tiles registered in (pinned) host memory; runtime moves them (copy_deps)
+    rt = vs.Runtime(lam=1)
+    A, B, C0, C = _matmul(rt, 512, 128, mask=1 << vs.VS_V_TC_3XTF32, host=True)
+    assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-5
+    st = rt.vs_stats()
+    tile = 128 * 128 * 4
+    assert st.input_tx_bytes == 3 * 16 * tile           # each A, B, C tile in once (R25)
+    assert st.output_tx_bytes == 16 * tile              # written C tiles flushed home
+    rt.close()
+
+
+def test_matmul_f64_family(gpu):
+    rt = vs.Runtime(lam=1)
+    mask = 1 << vs.VS_V_DFMA_F64
+    A, B, C0, C = _matmul(rt, 512, 128, dtype=vs.VS_F64, mask=mask)
+    assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-12
+    rt.close()
+
+
+def _cholesky(rt, N, b, mask=F32_MASK, seed=2, dtype=vs.VS_F32):
+    torch = _torch()
+    nt = N // b
+    types = rt.vs_register_builtins(dtype, mask)
+    npdt = np.float32 if dtype == vs.VS_F32 else np.float64
+    A = vsgen.spd(seed, N, npdt)
+    T = _tiles_dev(A, b)
+    ids = {}
+    nbytes = b * b * T.element_size()
+    for i in range(nt):
+        for j in range(i + 1):
+            ids[i * nt + j] = rt.vs_data_register(T[i, j].data_ptr(), 0, nbytes)
+    rt.vs_app_cholesky(types, nt, ids)
+    rt.vs_wait_all()
+    torch.cuda.synchronize()
+    return A, np.tril(vsgen.from_tiles(T.cpu().numpy()))
+
+
+def test_cfg2_cholesky_versioning(gpu):
+    # cfg2: Cholesky N=4096 SPD fp32, 512x512 tiles, 3 versions per task, lambda = 3.
+    # Oracle on the leading 2048 block (L[:k,:k] = chol(A[:k,:k])) + full-size residual.
+    rt = vs.Runtime(lam=3)
+    A, L = _cholesky(rt, 4096, 512)
+    k = 2048
+    Lk, info = oracle.cholesky(A[:k, :k])
+    assert info == 0
+    lo, slo = np.tril_indices(k), np.tril_indices(k, -1)
+    assert oracle.relF(L[:k, :k][lo], Lk[lo]) <= 1e-5
+    assert oracle.relF(L[:k, :k][slo], Lk[slo]) <= 1e-5
+    rng = np.random.default_rng(0)
+    A64, L64 = A.astype(np.float64), L.astype(np.float64)
+    for _ in range(4):
+        x = rng.standard_normal(4096)
+        r = A64 @ x - L64 @ (L64.T @ x)
+        assert np.linalg.norm(r) / np.linalg.norm(A64 @ x) <= 1e-5
+    gs = {g["type_name"]: g for g in rt.vs_group_stats()}
+    assert not gs["POTRF.f32"]["reliable"] and sum(gs["POTRF.f32"]["n"]) == 8     # L496-501
+    assert gs["GEMM_NT.f32"]["reliable"] and sum(gs["GEMM_NT.f32"]["n"]) == 56
+    rt.close()
+
+
+def test_cholesky_not_spd_sticky(gpu):
+    torch = _torch()
+    rt = vs.Runtime(lam=1)
+    types = rt.vs_register_builtins(vs.VS_F32, 1 << vs.VS_V_SIMT_F32)
+    b, nt = 128, 2
+    A = np.eye(256, dtype=np.float32)
+    A[200, 200] = -5.0
+    T = _tiles_dev(A, b)
+    ids = {i * nt + j: rt.vs_data_register(T[i, j].data_ptr(), 0, b * b * 4) for i in range(nt) for j in range(i + 1)}
+    rt.vs_app_cholesky(types, nt, ids)
+    with pytest.raises(vs.VSError) as e:
+        rt.vs_wait_all()
+    assert e.value.code == vs.VS_E_NOT_SPD
+    st = rt.vs_stats()
+    assert st.error_info == 200 - 128 + 1             # pivot within the failing tile
+    rt.close()
+    torch.cuda.synchronize()
+
+
+def test_replay_mode_bit_exact_outputs(gpu):
+    # P8: same timing table -> same decisions and bit-identical tiles across runs.
+    torch = _torch()
+    outs, hashes = [], []
+    for _ in range(2):
+        rt = vs.Runtime(vs.vs_config_default(lam=2, replay=1))
+        types = rt.vs_register_builtins(vs.VS_F32, F32_MASK)
+        nbytes = 256 * 256 * 4
+        for ti, sz in ((vs.VS_T_POTRF, nbytes), (vs.VS_T_TRSM, 2 * nbytes), (vs.VS_T_SYRK, 2 * nbytes),
+                       (vs.VS_T_GEMM_NT, 3 * nbytes)):
+            for v, d in enumerate((900, 300, 1500)):
+                rt.vs_replay_set(types[ti], sz, v, d + 17 * ti)
+        A = vsgen.spd(5, 1024)
+        T = _tiles_dev(A, 256)
+        ids = {i * 4 + j: rt.vs_data_register(T[i, j].data_ptr(), 0, nbytes) for i in range(4) for j in range(i + 1)}
+        rt.vs_app_cholesky(types, 4, ids)
+        rt.vs_wait_all()
+        torch.cuda.synchronize()
+        outs.append(T.cpu().numpy())
+        hashes.append(rt.vs_decision_log_hash())
+        rt.close()
+    assert hashes[0] == hashes[1]
+    assert np.array_equal(outs[0].view(np.uint32), outs[1].view(np.uint32))

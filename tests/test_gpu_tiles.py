@@ -1,0 +1,164 @@
+"""GPU parity of every built-in tile task version against the CPU oracle, through the C ABI
+(vs_tile_run).  Gates (BASELINE.json north star): relF <= 1e-5 for the fp32 class,
+<= 1e-12 for fp64; bit-exact where the arithmetic fixes the result (P1, P2, P6)."""
+import numpy as np
+import pytest
+
+import oracle
+import paper_conf_ipps_planasbal13_b200 as vs
+import vsgen
+
+pytestmark = pytest.mark.gpu
+
+F32_VERSIONS = [vs.VS_V_SIMT_F32, vs.VS_V_TC_3XTF32, vs.VS_V_F64IN_F32IO]
+F64_VERSIONS = [vs.VS_V_DFMA_F64]
+SIZES = [64, 128, 192, 320, 512]
+
+
+def _torch():
+    import torch
+    return torch
+
+
+def _dev(a):
+    torch = _torch()
+    return torch.from_numpy(np.ascontiguousarray(a)).cuda()
+
+
+def _host(t):
+    _torch().cuda.synchronize()
+    return t.cpu().numpy()
+
+
+def _run(ttype, version, b, arrays, info=None):
+    ts = [_dev(a) for a in arrays]
+    dinfo = info.data_ptr() if info is not None else 0
+    vs.vs_tile_run(ttype, version, b, [t.data_ptr() for t in ts], dinfo)
+    return [_host(t) for t in ts]
+
+
+def _gate(version):
+    return 1e-12 if version in (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64) else 1e-5
+
+
+def _dt(version):
+    return np.float64 if version in (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64) else np.float32
+
+
+# ------------------------------------------------------------------ generator
+def test_device_generator_bit_identical(gpu):
+    torch = _torch()
+    for tile_b in (0, 32):
+        out = torch.empty(96 * 64, dtype=torch.float32, device="cuda")
+        vs.vs_gen_uniform(7, 96, 64, vs.VS_F32, tile_b, out.data_ptr())
+        ref = vsgen.uniform(7, 96, 64)
+        if tile_b:
+            ref = vsgen.to_tiles(ref, tile_b)
+        assert np.array_equal(_host(out).reshape(ref.shape), ref)
+    out = torch.empty(320 * 320, dtype=torch.float64, device="cuda")
+    vs.vs_gen_spd(9, 320, vs.VS_F64, 64, out.data_ptr())
+    ref = vsgen.to_tiles(vsgen.spd(9, 320, np.float64), 64)
+    assert np.array_equal(_host(out).reshape(ref.shape), ref)
+    out = torch.empty(512 * 512, dtype=torch.float32, device="cuda")
+    vs.vs_gen_spd(2, 512, vs.VS_F32, 0, out.data_ptr())
+    assert np.array_equal(_host(out).reshape(512, 512), vsgen.spd(2, 512))
+
+
+# ------------------------------------------------------------------ matmul / gemm / syrk
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("b", SIZES)
+def test_matmul_tile(gpu, version, b):
+    dt = _dt(version)
+    A, B, C0 = (vsgen.uniform(100 + i, b, b, dt) for i in range(3))
+    (_, _, C) = _run(vs.VS_T_MATMUL, version, b, [A, B, C0])
+    ref = oracle.matmul(A, B, C0)
+    assert oracle.relF(C, ref) <= _gate(version)
+
+
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("b", SIZES)
+def test_gemm_nt_and_syrk_tiles(gpu, version, b):
+    dt = _dt(version)
+    A, B, C0 = (vsgen.uniform(200 + i, b, b, dt) for i in range(3))
+    (_, _, C) = _run(vs.VS_T_GEMM_NT, version, b, [A, B, C0])
+    assert oracle.relF(C, oracle.gemm_nt(A, B, C0)) <= _gate(version)
+    (_, S) = _run(vs.VS_T_SYRK, version, b, [A, C0])
+    ref = oracle.syrk(A, C0)
+    lo = np.tril_indices(b)
+    assert oracle.relF(S[lo], ref[lo]) <= _gate(version)
+    up = np.triu_indices(b, 1)
+    assert np.array_equal(S[up], C0[up])          # strict upper untouched (R7)
+
+
+def test_simt_f32_bit_exact_fig1_fmaf(gpu):
+    # P6: simt_f32 == Fig 1 with fmaf, ascending k, from C_in — bit for bit.
+    b = 192
+    A, B, C0 = (vsgen.uniform(300 + i, b, b) for i in range(3))
+    (_, _, C) = _run(vs.VS_T_MATMUL, vs.VS_V_SIMT_F32, b, [A, B, C0])
+    ref = oracle.matmul_tiled_fmaf_f32(A[None, None], B[None, None], C0[None, None])[0, 0]
+    assert np.array_equal(C.view(np.uint32), ref.view(np.uint32))
+    (_, _, G) = _run(vs.VS_T_GEMM_NT, vs.VS_V_SIMT_F32, b, [A, B, C0])
+    assert np.array_equal(G.view(np.uint32), oracle.gemm_nt_fmaf_f32(A, B, C0).view(np.uint32))
+
+
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+def test_integer_inputs_exact(gpu, version):
+    # P1: integer inputs -> exact results in every version (|C| < 2^24, ints exact in TF32).
+    b = 256
+    dt = _dt(version)
+    A, B, C0 = (vsgen.int_matrix(400 + i, b, b, dtype=dt) for i in range(3))
+    (_, _, C) = _run(vs.VS_T_MATMUL, version, b, [A, B, C0])
+    exact = C0.astype(np.int64) + A.astype(np.int64) @ B.astype(np.int64)
+    assert np.array_equal(C.astype(np.int64), exact)
+    (_, _, G) = _run(vs.VS_T_GEMM_NT, version, b, [A, B, C0])
+    assert np.array_equal(G.astype(np.int64), C0.astype(np.int64) - A.astype(np.int64) @ B.astype(np.int64).T)
+
+
+# ------------------------------------------------------------------ trsm / potrf
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("b", [64, 128, 192, 512])
+def test_trsm_tile(gpu, version, b):
+    dt = _dt(version)
+    Lfull, _ = oracle.cholesky(vsgen.spd(500 + b, b, np.float64))
+    L = Lfull.astype(dt)
+    X0 = vsgen.uniform(501, b, b, dt)
+    (_, X) = _run(vs.VS_T_TRSM, version, b, [L, X0])
+    assert oracle.relF(X, oracle.trsm(L, X0)) <= _gate(version)
+
+
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("b", [64, 128, 192, 512])
+def test_potrf_tile(gpu, version, b):
+    torch = _torch()
+    dt = _dt(version)
+    A = vsgen.spd(600 + b, b, dt)
+    junk = A.copy()
+    junk[np.triu_indices(b, 1)] = 777.0
+    info = torch.zeros(1, dtype=torch.int32, device="cuda")
+    (L,) = _run(vs.VS_T_POTRF, version, b, [junk], info)
+    assert int(info.item()) == 0
+    ref, _ = oracle.cholesky(A)
+    lo = np.tril_indices(b)
+    slo = np.tril_indices(b, -1)
+    assert oracle.relF(L[lo], ref[lo]) <= _gate(version)
+    assert oracle.relF(L[slo], ref[slo]) <= 5 * _gate(version)     # R23 strict-lower gate
+    assert np.all(L[np.triu_indices(b, 1)] == 777.0)                  # R7
+
+
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+def test_potrf_integer_L0_exact_and_info(gpu, version):
+    torch = _torch()
+    dt = _dt(version)
+    b = 128
+    L0 = vsgen.int_lower(11, b)
+    A = (L0.astype(np.int64) @ L0.T.astype(np.int64)).astype(dt)
+    info = torch.zeros(1, dtype=torch.int32, device="cuda")
+    (L,) = _run(vs.VS_T_POTRF, version, b, [A], info)
+    assert int(info.item()) == 0
+    assert np.array_equal(np.tril(L).astype(np.float64), L0)
+    # non-SPD: pivot 70 (1-based) is the first non-positive one
+    bad = np.eye(b, dtype=dt) * 4
+    bad[69, 69] = -1.0
+    info.zero_()
+    _run(vs.VS_T_POTRF, version, b, [bad], info)
+    assert int(info.item()) == 70
