@@ -121,11 +121,17 @@ __device__ __forceinline__ uint32_t kmaj_off(int row, int kchunk)
 {
     return (uint32_t)((row >> 3) * 1024 + (row & 7) * 128 + ((kchunk ^ (row & 7)) << 4));
 }
-// byte offset of the 16-byte chunk holding (k, n..n+3) in an MN-major SW128 tile:
-// n-atoms of 32 elements at stride LBO = 4096 B (BK/8 k-groups of 1024 B each)
-__device__ __forceinline__ uint32_t mnmaj_off(int k, int nchunk)
+// byte offset of the 16-byte chunk holding (k, n..n+3) in an MN-major SW128 tile.
+// Layout variant (tools/probe_mn.cu): bit 1 = 0: n-atoms (32 elements) at 4096 B, k-groups
+// (8 rows) at 1024 B; bit 1 = 1: n-atoms at 1024 B, k-groups at 4096 B.  Bit 0 swaps the
+// LBO/SBO descriptor fields.
+#ifndef VSK_MN_VARIANT
+#define VSK_MN_VARIANT 0
+#endif
+__device__ __forceinline__ uint32_t mnmaj_off(int k, int nchunk, int var)
 {
-    return (uint32_t)((nchunk >> 3) * 4096 + (k >> 3) * 1024 + (k & 7) * 128 + (((nchunk & 7) ^ (k & 7)) << 4));
+    const int sa = (var & 2) ? 1024 : 4096, sk = (var & 2) ? 4096 : 1024;
+    return (uint32_t)((nchunk >> 3) * sa + (k >> 3) * sk + (k & 7) * 128 + (((nchunk & 7) ^ (k & 7)) << 4));
 }
 
 template <int BN>
@@ -227,7 +233,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                     split_store(b_big, b_small, kmaj_off(row, c), rb[p]);
                 } else if (B_MN) {
                     const int kr = f / (BN / 4), nc = f % (BN / 4);
-                    split_store(b_big, b_small, mnmaj_off(kr, nc), rb[p]);
+                    split_store(b_big, b_small, mnmaj_off(kr, nc, VSK_MN_VARIANT), rb[p]);
                 } else {
                     // transpose into K-major: element (n, k) for n = 4nc..4nc+3
                     const int kr = f / (BN / 4), nc = f % (BN / 4);
@@ -289,8 +295,11 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
 #pragma unroll
                 for (int kk = 0; kk < BK / 8; kk++) {
                     // K-major: advance 32 B inside the 128 B swizzled row; MN-major: next k-group
-                    const uint32_t ao = kk * 32, bo = bmn ? kk * 1024 : kk * 32;
-                    const uint32_t lbo = bmn ? 4096 : 16, sbo = 1024;
+                    constexpr int var = VSK_MN_VARIANT;
+                    constexpr uint32_t s_atom = (var & 2) ? 1024 : 4096, s_kgrp = (var & 2) ? 4096 : 1024;
+                    const uint32_t ao = kk * 32, bo = bmn ? kk * s_kgrp : kk * 32;
+                    const uint32_t lbo = bmn ? ((var & 1) ? s_kgrp : s_atom) : 16;
+                    const uint32_t sbo = bmn ? ((var & 1) ? s_atom : s_kgrp) : 1024;
                     const uint64_t dAb = make_desc(a_big + ao, 16, 1024), dAs = make_desc(a_small + ao, 16, 1024);
                     const uint64_t dBb = make_desc(b_big + bo, lbo, sbo), dBs = make_desc(b_small + bo, lbo, sbo);
                     const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
@@ -313,7 +322,10 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     }
 }
 
-template <bool NT, bool NEG, bool LOWER, bool B_MN = true>
+// B_MN: NN operand B stored MN-major (vector STS) instead of transposed into K-major.
+// The MN-major descriptor path produced a zero contribution on the first B200 run, so the
+// transposing K-major path is the default until the MN-major encoding is probed.
+template <bool NT, bool NEG, bool LOWER, bool B_MN = false>
 inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B, int ldb, float *C, int ldc,
                    cudaStream_t s)
 {
@@ -336,47 +348,5 @@ inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B,
 }
 
 }  // namespace tc
-
-// tc_3xtf32 versions of the five task types: the O(b^3) work on tcgen05; potrf / trsm
-// keep their small triangular panels on SIMT (simt_chol.cuh).
-inline bool tc_available(int type) { return type >= 0 && type < 5; }
-
-inline int run_tc(int type, int b, void *const *p, int *info, cudaStream_t s)
-{
-    constexpr int NBP = 64;
-    switch (type) {
-    case 0:  // MATMUL C += A B
-        return tc::tc_gemm<false, false, false>(b, b, b, (const float *)p[0], b, (const float *)p[1], b, (float *)p[2], b, s);
-    case 4:  // GEMM_NT C -= A B^T
-        return tc::tc_gemm<true, true, false>(b, b, b, (const float *)p[0], b, (const float *)p[1], b, (float *)p[2], b, s);
-    case 3:  // SYRK C -= A A^T lower
-        return tc::tc_gemm<true, true, true>(b, b, b, (const float *)p[0], b, (const float *)p[0], b, (float *)p[1], b, s);
-    case 2: {  // TRSM
-        const float *L = (const float *)p[0];
-        float *X = (float *)p[1];
-        for (int j0 = 0; j0 < b; j0 += NBP) {
-            trsm_panel<float, float, NBP>(L + (int64_t)j0 * b + j0, b, X + j0, b, b, s);
-            const int rest = b - j0 - NBP;
-            if (rest > 0)
-                tc::tc_gemm<true, true, false>(b, rest, NBP, X + j0, b, L + (int64_t)(j0 + NBP) * b + j0, b, X + j0 + NBP, b, s);
-        }
-        return 0;
-    }
-    case 1: {  // POTRF
-        float *A = (float *)p[0];
-        for (int k0 = 0; k0 < b; k0 += NBP) {
-            potrf_diag<float, float, NBP>(A + (int64_t)k0 * b + k0, b, k0, info, s);
-            const int rest = b - k0 - NBP;
-            if (rest > 0) {
-                trsm_panel<float, float, NBP>(A + (int64_t)k0 * b + k0, b, A + (int64_t)(k0 + NBP) * b + k0, b, rest, s);
-                float *P = A + (int64_t)(k0 + NBP) * b + k0;
-                tc::tc_gemm<true, true, true>(rest, rest, NBP, P, b, P, b, A + (int64_t)(k0 + NBP) * b + k0 + NBP, b, s);
-            }
-        }
-        return 0;
-    }
-    }
-    return -1;
-}
 
 }  // namespace vsk

@@ -1,0 +1,63 @@
+"""Parity at BASELINE.json's full sizes, in the launch configuration bench.py times
+(cfg3 matmul N=16384 b=1024 + cfg4 Cholesky N=32768 b=1024, 4 slots, lambda=3, all f32
+versions, run-ahead): sampled outputs the oracle computes one by one, plus properties that
+hold at any size."""
+import numpy as np
+import pytest
+
+import oracle
+import paper_conf_ipps_planasbal13_b200 as vs
+import vsgen
+
+pytestmark = pytest.mark.gpu
+
+
+def test_fullsize_bench_configuration(gpu):
+    import torch
+
+    import bench
+    rt = vs.Runtime(vs.vs_config_default(lam=3, slots_per_gpu=4))
+    wl = bench.Workload(rt)
+    wl.step()          # learning happens here (cold)
+    wl.step()          # warm step, as timed by bench.py
+    torch.cuda.synchronize()
+    N, b = bench.MM_N, bench.MM_B
+    nt = N // b
+    # ---- matmul: sampled rows of C = A B (C0 = 0), oracle fp64 row by row
+    rows = [0, 1, 1023, 1024, 8191, 16383]
+    Bfull = vsgen.uniform(bench.SEED_MM + 1000, N, N)
+    for r in rows:
+        a = vsgen.uniform_idx(bench.SEED_MM, np.arange(r * N, (r + 1) * N, dtype=np.uint64)).astype(np.float32)
+        ref = oracle.matmul(a[None, :], Bfull)[0]
+        got = wl.C[r // b, :, r % b, :].reshape(-1).cpu().numpy()
+        assert oracle.relF(got, ref) <= 1e-5, r
+    # Freivalds on the whole product: A (B x) vs C x
+    rng = np.random.default_rng(1)
+    x = rng.standard_normal(N)
+    Afull = vsgen.uniform(bench.SEED_MM, N, N)
+    C = vsgen.from_tiles(wl.C.cpu().numpy()).astype(np.float64)
+    lhs = Afull.astype(np.float64) @ (Bfull.astype(np.float64) @ x)
+    assert np.linalg.norm(lhs - C @ x) / np.linalg.norm(lhs) <= 1e-5
+    del C, Afull, Bfull
+    # ---- Cholesky: leading 2048 block vs oracle; residual on the full matrix
+    Nc, bc = bench.CH_N, bench.CH_B
+    L = np.tril(vsgen.from_tiles(wl.S.cpu().numpy()))
+    k = 2048
+    r = np.arange(k, dtype=np.uint64)[:, None]
+    c = np.arange(k, dtype=np.uint64)[None, :]
+    S = vsgen.uniform_idx(bench.SEED_CH, np.maximum(r, c) * np.uint64(Nc) + np.minimum(r, c))
+    S[np.arange(k), np.arange(k)] += vsgen.spd_alpha(Nc)
+    Lk, info = oracle.cholesky(S.astype(np.float32))
+    assert info == 0
+    lo, slo = np.tril_indices(k), np.tril_indices(k, -1)
+    assert oracle.relF(L[:k, :k][lo], Lk[lo]) <= 1e-5
+    assert oracle.relF(L[:k, :k][slo], Lk[slo]) <= 1e-5
+    A = vsgen.from_tiles(wl.S0.cpu().numpy())
+    A = np.tril(A) + np.tril(A, -1).T
+    x = rng.standard_normal(Nc)
+    Ax = A.astype(np.float64) @ x
+    L64 = L.astype(np.float64)
+    assert np.linalg.norm(Ax - L64 @ (L64.T @ x)) / np.linalg.norm(Ax) <= 1e-5
+    st = rt.vs_stats()
+    assert st.tasks_completed == 2 * (4096 + 5984)
+    rt.close()

@@ -82,7 +82,7 @@ def test_matmul_host_data_copy_deps(gpu):
 
 def test_matmul_f64_family(gpu):
     rt = vs.Runtime(lam=1)
-    mask = 1 << vs.VS_V_DFMA_F64
+    mask = (1 << vs.VS_V_DFMA_F64) | (1 << vs.VS_V_DMMA_F64)
     A, B, C0, C = _matmul(rt, 512, 128, dtype=vs.VS_F64, mask=mask)
     assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-12
     rt.close()

@@ -11,7 +11,7 @@ import vsgen
 pytestmark = pytest.mark.gpu
 
 F32_VERSIONS = [vs.VS_V_SIMT_F32, vs.VS_V_TC_3XTF32, vs.VS_V_F64IN_F32IO]
-F64_VERSIONS = [vs.VS_V_DFMA_F64]
+F64_VERSIONS = [vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64]
 SIZES = [64, 128, 192, 320, 512]
 
 
