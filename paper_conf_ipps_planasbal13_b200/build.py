@@ -23,7 +23,9 @@ def _sources():
 
 
 def _headers():
-    return sorted(glob.glob(os.path.join(CSRC, "**", "*.h*"), recursive=True) + [os.path.join(ROOT, "include", "vsched.h")])
+    pats = ("*.h", "*.hpp", "*.cuh")
+    hs = [h for p in pats for h in glob.glob(os.path.join(CSRC, "**", p), recursive=True)]
+    return sorted(hs + [os.path.join(ROOT, "include", "vsched.h")])
 
 
 def _compile(src: str, verbose: bool) -> str:
