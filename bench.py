@@ -263,6 +263,9 @@ def main():
     ap.add_argument("--small", action="store_true", help="cfg1/cfg2-sized smoke of the bench itself")
     ap.add_argument("--only", choices=["mm", "ch", "both"], default="both")
     ap.add_argument("--dump-log", default="")
+    ap.add_argument("--table-dump", default="", help="write the learned TaskVersionSets after warm-up")
+    ap.add_argument("--table-load", default="", help="warm start from a table (NEXT-2 hints)")
+    ap.add_argument("--replay", action="store_true", help="decisions from the loaded table (profiling runs)")
     args = ap.parse_args()
     rank = int(os.environ.get("RANK", "0"))
     world = int(os.environ.get("WORLD_SIZE", "1"))
@@ -284,9 +287,19 @@ def main():
 
     mm_n, mm_b, ch_n, ch_b = (MM_N, MM_B, CH_N, CH_B) if not args.small else (1024, 256, 4096, 512)
     with_mm, with_ch = args.only in ("mm", "both"), args.only in ("ch", "both")
-    cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0)
+    cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0)
     rt = vs.Runtime(cfg)
     wl = Workload(rt, mm_n, mm_b, ch_n, ch_b, host=False, seed_off=rank, with_mm=with_mm, with_ch=with_ch)
+    if args.table_load:
+        rt.vs_table_load(args.table_load)
+        if args.replay:          # replay durations = the loaded means
+            for line in open(args.table_load):
+                tn, nb, vn, mean, n = line.split()
+                for ti in wl.types:
+                    if vs.lib().vs_type_name(rt.h, ti).decode() == tn:
+                        vi = [vs.lib().vs_version_name(rt.h, ti, v).decode() for v in range(8)
+                              if vs.lib().vs_version_name(rt.h, ti, v)].index(vn)
+                        rt.vs_replay_set(ti, int(nb), vi, int(mean))
 
     # warm-up (the first step includes the learning phase: "cold")
     t0 = time.perf_counter()
@@ -294,6 +307,8 @@ def main():
     cold_ms = (time.perf_counter() - t0) * 1e3
     for _ in range(args.warmup - 1):
         wl.step()
+    if args.table_dump:
+        rt.vs_table_dump(args.table_dump)
     rt.vs_decision_log_clear()
     st0 = rt.vs_stats()
 

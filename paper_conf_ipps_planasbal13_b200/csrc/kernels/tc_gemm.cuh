@@ -5,20 +5,24 @@
 //
 // 3xTF32: every fp32 operand x is split into big = rna_tf32(x) and small = x - big
 // (exact in fp32), and D += Ab*Bb + Ab*Bs + As*Bb is accumulated in fp32 in TMEM by
-// three tcgen05.mma.kind::tf32 per k-step (the dropped As*Bs term is < 2^-22 |a||b|).
+// three tcgen05.mma.kind::tf32 per 8-wide k-step (the dropped As*Bs term is
+// < 2^-22 |a||b|).  The sign s is the instruction descriptor's negate-A bit.
 //
-// Structure (one 128 x BN output tile per CTA, cta_group::1):
-//   warps 0-3  producers: LDG.128 fp32 k-blocks (32 wide) -> split in registers ->
-//              STS into 128B-swizzled K-major (A, and B in NT form) or MN-major (B in
-//              NN form) UMMA layouts; fence.proxy.async; mbarrier arrive (full[s]).
-//              The next k-block's loads are in flight while the current one is stored.
-//   warp 4     TMEM allocator + MMA issuer: one elected lane waits full[s], issues
-//              3 x (BK/8) MMAs, tcgen05.commit -> empty[s]; after the last k-block,
+// Structure (one 128 x BN output tile per CTA, cta_group::1, UMMA M=128, N=BN):
+//   warps 0-7  producers (256 threads): LDG.128 of fp32 k-blocks (32 wide) two k-blocks
+//              ahead in registers -> split -> STS.128 into 128B-swizzled K-major UMMA
+//              layouts (A; B in NT form; B in NN form after a 4x4 register transpose so
+//              the store stays a conflict-free 16-byte vector) -> fence.proxy.async ->
+//              mbarrier arrive (full[s]).  STAGES smem stages of {A,B} x {big,small}.
+//   warp 8     TMEM allocator + MMA issuer: one lane waits full[s], issues 3 x (BK/8)
+//              tcgen05.mma, tcgen05.commit -> empty[s]; after the last k-block,
 //              commit -> acc_full.
-//   warps 0-3  epilogue: tcgen05.ld 32x32b.x32 (warp w owns TMEM lanes 32w..32w+31 =
-//              tile rows), C += acc with fp32 round-to-nearest, vector stores.
+//   warps 0-7  epilogue: warp w reads TMEM lanes 32(w%4).. (tile rows) and column half
+//              w/4 with tcgen05.ld 32x32b.x32, C += acc (fp32 RN), vector stores.
 // LOWER (syrk / potrf update): CTAs strictly above the diagonal exit; diagonal tiles
 // store only j <= i.
+// The MN-major B encoding (no transpose) was probed on B200 (tools/probe_mn.cu): with the
+// B-major bit set the tf32 MMA contributed nothing, so NN B is transposed in registers.
 #pragma once
 #include <cuda_runtime.h>
 #include <stdint.h>
@@ -28,8 +32,8 @@
 namespace vsk {
 namespace tc {
 
-constexpr int BM = 128, BK = 32, STAGES = 3;
-constexpr int NPROD = 128;  // producer / epilogue threads (warps 0-3)
+constexpr int BM = 128, BK = 32;
+constexpr int NPROD = 256;  // producer / epilogue threads (warps 0-7)
 constexpr int NTHREADS = NPROD + 32;
 
 __device__ __forceinline__ uint32_t smem_u32(const void *p) { return (uint32_t)__cvta_generic_to_shared(p); }
@@ -116,41 +120,45 @@ __device__ __forceinline__ void tmem_ld32(uint32_t taddr, float (&v)[32])
     for (int i = 0; i < 32; i++) v[i] = __uint_as_float(r[i]);
 }
 
-// byte offset of element (row, k) in a K-major SW128 tile (rows of 32 fp32 = 128 B)
+// byte offset of the 16-byte chunk (row, k = 4*kchunk .. 4*kchunk+3) in a K-major SW128
+// tile: rows of 32 fp32 = 128 B, 8-row atoms of 1024 B, chunk index XOR (row & 7).
 __device__ __forceinline__ uint32_t kmaj_off(int row, int kchunk)
 {
     return (uint32_t)((row >> 3) * 1024 + (row & 7) * 128 + ((kchunk ^ (row & 7)) << 4));
 }
-// byte offset of the 16-byte chunk holding (k, n..n+3) in an MN-major SW128 tile.
-// Layout variant (tools/probe_mn.cu): bit 1 = 0: n-atoms (32 elements) at 4096 B, k-groups
-// (8 rows) at 1024 B; bit 1 = 1: n-atoms at 1024 B, k-groups at 4096 B.  Bit 0 swaps the
-// LBO/SBO descriptor fields.
-#ifndef VSK_MN_VARIANT
-#define VSK_MN_VARIANT 0
-#endif
-__device__ __forceinline__ uint32_t mnmaj_off(int k, int nchunk, int var)
-{
-    const int sa = (var & 2) ? 1024 : 4096, sk = (var & 2) ? 4096 : 1024;
-    return (uint32_t)((nchunk >> 3) * sa + (k >> 3) * sk + (k & 7) * 128 + (((nchunk & 7) ^ (k & 7)) << 4));
-}
 
 template <int BN>
-struct Smem {
+struct Cfg {
+    static constexpr int STAGES = BN >= 256 ? 2 : 3;
     static constexpr int A_BYTES = BM * BK * 4;   // 16 KB
     static constexpr int B_BYTES = BN * BK * 4;
     static constexpr int STAGE = 2 * A_BYTES + 2 * B_BYTES;
-    static constexpr int TOTAL = STAGES * STAGE + 1024 /*align*/ + 256 /*barriers*/;
+    static constexpr int SMEM = STAGES * STAGE + 1024 /*align*/ + 256 /*barriers*/;
+    static constexpr int APER = BM * BK / 4 / NPROD;        // A float4 per thread (4)
+    static constexpr int BPER = BN * BK / 4 / NPROD;        // B float4 per thread (BN/32)
 };
 
-template <int BN, bool NT, bool NEG, bool LOWER, bool B_MN>
+__device__ __forceinline__ float4 split_big(float4 v)
+{
+    return make_float4(to_tf32(v.x), to_tf32(v.y), to_tf32(v.z), to_tf32(v.w));
+}
+__device__ __forceinline__ void store_split(uint8_t *big, uint8_t *small, uint32_t off, float4 v)
+{
+    const float4 b = split_big(v);
+    *reinterpret_cast<float4 *>(big + off) = b;
+    *reinterpret_cast<float4 *>(small + off) = make_float4(v.x - b.x, v.y - b.y, v.z - b.z, v.w - b.w);
+}
+
+template <int BN, bool NT, bool NEG, bool LOWER>
 __global__ void __launch_bounds__(NTHREADS, 1)
 tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const float *__restrict__ B, int ldb,
                float *__restrict__ C, int ldc)
 {
-    using S = Smem<BN>;
+    using G = Cfg<BN>;
+    constexpr int STAGES = G::STAGES;
     extern __shared__ uint8_t smem_raw[];
     uint8_t *smem = (uint8_t *)(((uintptr_t)smem_raw + 1023) & ~(uintptr_t)1023);
-    uint64_t *full = (uint64_t *)(smem + STAGES * S::STAGE);
+    uint64_t *full = (uint64_t *)(smem + STAGES * G::STAGE);
     uint64_t *empty = full + STAGES;
     uint64_t *acc_full = empty + STAGES;
     uint32_t *tmem_slot = (uint32_t *)(acc_full + 1);
@@ -168,7 +176,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
         mbar_init(acc_full, 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     }
-    if (warp == 4) {
+    if (warp == NPROD / 32) {
         asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(tmem_slot)),
                      "r"((uint32_t)BN));
         asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
@@ -178,130 +186,127 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     tc_fence_after();
     const uint32_t tmem = *tmem_slot;
 
-    if (warp < 4) {
+    if (warp < NPROD / 32) {
         // ------------------------------------------------------------ producers
         const int t = threadIdx.x;
-        constexpr int APER = BM * BK / 4 / NPROD;  // float4 per thread (8)
-        constexpr int BPER = BN * BK / 4 / NPROD;
-        float4 ra[APER], rb[BPER];
-        auto load = [&](int kb) {
+        constexpr int APER = G::APER, BPER = G::BPER;
+        const float4 z4 = make_float4(0.f, 0.f, 0.f, 0.f);
+        auto load = [&](float4 (&ra)[APER], float4 (&rb)[BPER], int kb) {
             const int k0 = kb * BK;
 #pragma unroll
             for (int p = 0; p < APER; p++) {
                 const int f = t + p * NPROD, row = f >> 3, c = f & 7;
-                ra[p] = (m0 + row < M) ? __ldg(reinterpret_cast<const float4 *>(A + (int64_t)(m0 + row) * lda + k0 + 4 * c))
-                                       : make_float4(0.f, 0.f, 0.f, 0.f);
+                ra[p] = (m0 + row < M) ? __ldg(reinterpret_cast<const float4 *>(A + (int64_t)(m0 + row) * lda + k0 + 4 * c)) : z4;
             }
+            if (NT) {
 #pragma unroll
-            for (int p = 0; p < BPER; p++) {
-                const int f = t + p * NPROD;
-                if (NT) {
-                    const int row = f >> 3, c = f & 7;
-                    rb[p] = (n0 + row < N) ? __ldg(reinterpret_cast<const float4 *>(B + (int64_t)(n0 + row) * ldb + k0 + 4 * c))
-                                           : make_float4(0.f, 0.f, 0.f, 0.f);
-                } else {
-                    const int kr = f / (BN / 4), nc = f % (BN / 4);
-                    rb[p] = (n0 + 4 * nc < N) ? __ldg(reinterpret_cast<const float4 *>(B + (int64_t)(k0 + kr) * ldb + n0 + 4 * nc))
-                                              : make_float4(0.f, 0.f, 0.f, 0.f);
+                for (int p = 0; p < BPER; p++) {
+                    const int f = t + p * NPROD, row = f >> 3, c = f & 7;
+                    rb[p] = (n0 + row < N) ? __ldg(reinterpret_cast<const float4 *>(B + (int64_t)(n0 + row) * ldb + k0 + 4 * c)) : z4;
+                }
+            } else {
+                // NN: 4 (k) x 4 (n) blocks; unit u -> kq = u / (BN/4), nq = u % (BN/4)
+#pragma unroll
+                for (int p = 0; p < BPER / 4; p++) {
+                    const int u = t + p * NPROD, kq = u / (BN / 4), nq = u % (BN / 4);
+                    const bool ok = n0 + 4 * nq < N;
+#pragma unroll
+                    for (int i = 0; i < 4; i++)
+                        rb[4 * p + i] = ok ? __ldg(reinterpret_cast<const float4 *>(B + (int64_t)(k0 + 4 * kq + i) * ldb + n0 + 4 * nq)) : z4;
                 }
             }
         };
-        auto split_store = [&](uint8_t *dst_big, uint8_t *dst_small, uint32_t off, float4 v) {
-            float4 b, s;
-            b.x = to_tf32(v.x); b.y = to_tf32(v.y); b.z = to_tf32(v.z); b.w = to_tf32(v.w);
-            s.x = v.x - b.x; s.y = v.y - b.y; s.z = v.z - b.z; s.w = v.w - b.w;
-            *reinterpret_cast<float4 *>(dst_big + off) = b;
-            *reinterpret_cast<float4 *>(dst_small + off) = s;
-        };
-        load(0);
-        for (int kb = 0; kb < nk; kb++) {
+        auto produce = [&](float4 (&ra)[APER], float4 (&rb)[BPER], int kb) {
             const int s = kb % STAGES;
             if (kb >= STAGES) mbar_wait(&empty[s], ((kb / STAGES) - 1) & 1);
-            uint8_t *st = smem + s * S::STAGE;
-            uint8_t *a_big = st, *a_small = st + S::A_BYTES;
-            uint8_t *b_big = st + 2 * S::A_BYTES, *b_small = b_big + S::B_BYTES;
+            uint8_t *st = smem + s * G::STAGE;
+            uint8_t *a_big = st, *a_small = st + G::A_BYTES;
+            uint8_t *b_big = st + 2 * G::A_BYTES, *b_small = b_big + G::B_BYTES;
 #pragma unroll
             for (int p = 0; p < APER; p++) {
                 const int f = t + p * NPROD, row = f >> 3, c = f & 7;
-                split_store(a_big, a_small, kmaj_off(row, c), ra[p]);
+                store_split(a_big, a_small, kmaj_off(row, c), ra[p]);
             }
+            if (NT) {
 #pragma unroll
-            for (int p = 0; p < BPER; p++) {
-                const int f = t + p * NPROD;
-                if (NT) {
-                    const int row = f >> 3, c = f & 7;
-                    split_store(b_big, b_small, kmaj_off(row, c), rb[p]);
-                } else if (B_MN) {
-                    const int kr = f / (BN / 4), nc = f % (BN / 4);
-                    split_store(b_big, b_small, mnmaj_off(kr, nc, VSK_MN_VARIANT), rb[p]);
-                } else {
-                    // transpose into K-major: element (n, k) for n = 4nc..4nc+3
-                    const int kr = f / (BN / 4), nc = f % (BN / 4);
-                    const float e[4] = {rb[p].x, rb[p].y, rb[p].z, rb[p].w};
+                for (int p = 0; p < BPER; p++) {
+                    const int f = t + p * NPROD, row = f >> 3, c = f & 7;
+                    store_split(b_big, b_small, kmaj_off(row, c), rb[p]);
+                }
+            } else {
 #pragma unroll
-                    for (int q = 0; q < 4; q++) {
-                        const int n = 4 * nc + q;
-                        const uint32_t off = kmaj_off(n, kr >> 2) + (kr & 3) * 4;
-                        const float bb = to_tf32(e[q]);
-                        *reinterpret_cast<float *>(b_big + off) = bb;
-                        *reinterpret_cast<float *>(b_small + off) = e[q] - bb;
-                    }
+                for (int p = 0; p < BPER / 4; p++) {
+                    const int u = t + p * NPROD, kq = u / (BN / 4), nq = u % (BN / 4);
+                    const float4 r0 = rb[4 * p], r1 = rb[4 * p + 1], r2 = rb[4 * p + 2], r3 = rb[4 * p + 3];
+                    // column n' of the 4x4 block = K-major 16-byte chunk of row n = 4nq+n'
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 0, kq), make_float4(r0.x, r1.x, r2.x, r3.x));
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 1, kq), make_float4(r0.y, r1.y, r2.y, r3.y));
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 2, kq), make_float4(r0.z, r1.z, r2.z, r3.z));
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 3, kq), make_float4(r0.w, r1.w, r2.w, r3.w));
                 }
             }
             fence_proxy_async();
             mbar_arrive(&full[s]);
-            if (kb + 1 < nk) load(kb + 1);
+        };
+        // two k-blocks of loads in flight (register double buffer, loop unrolled by 2)
+        float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
+        load(ra0, rb0, 0);
+        if (nk > 1) load(ra1, rb1, 1);
+        for (int kb = 0; kb < nk; kb += 2) {
+            produce(ra0, rb0, kb);
+            if (kb + 2 < nk) load(ra0, rb0, kb + 2);
+            if (kb + 1 < nk) {
+                produce(ra1, rb1, kb + 1);
+                if (kb + 3 < nk) load(ra1, rb1, kb + 3);
+            }
         }
 
         // ------------------------------------------------------------ epilogue
         mbar_wait(acc_full, 0);
         tc_fence_after();
-        const int row = m0 + warp * 32 + lane;
+        const int q = warp & 3, h = warp >> 2;
+        const int row = m0 + q * 32 + lane;
 #pragma unroll 1
-        for (int c = 0; c < BN / 32; c++) {
+        for (int c = 0; c < BN / 64; c++) {
+            const int col0 = h * (BN / 2) + c * 32;
             float v[32];
-            tmem_ld32(tmem + ((uint32_t)(warp * 32) << 16) + (uint32_t)(c * 32), v);
+            tmem_ld32(tmem + ((uint32_t)(q * 32) << 16) + (uint32_t)col0, v);
             if (row < M) {
-                float *crow = C + (int64_t)row * ldc + n0 + c * 32;
+                float *crow = C + (int64_t)row * ldc + n0 + col0;
 #pragma unroll
-                for (int q = 0; q < 8; q++) {
-                    const int col = n0 + c * 32 + 4 * q;
+                for (int j = 0; j < 8; j++) {
+                    const int col = n0 + col0 + 4 * j;
                     if (col >= N) break;
-                    float4 o = *reinterpret_cast<float4 *>(crow + 4 * q);
+                    float4 o = *reinterpret_cast<float4 *>(crow + 4 * j);
                     if (LOWER && col + 3 > row) {
-                        if (col + 0 <= row) o.x += v[4 * q + 0];
-                        if (col + 1 <= row) o.y += v[4 * q + 1];
-                        if (col + 2 <= row) o.z += v[4 * q + 2];
-                        if (col + 3 <= row) o.w += v[4 * q + 3];
+                        if (col + 0 <= row) o.x += v[4 * j + 0];
+                        if (col + 1 <= row) o.y += v[4 * j + 1];
+                        if (col + 2 <= row) o.z += v[4 * j + 2];
+                        if (col + 3 <= row) o.w += v[4 * j + 3];
                     } else {
-                        o.x += v[4 * q + 0]; o.y += v[4 * q + 1]; o.z += v[4 * q + 2]; o.w += v[4 * q + 3];
+                        o.x += v[4 * j + 0]; o.y += v[4 * j + 1]; o.z += v[4 * j + 2]; o.w += v[4 * j + 3];
                     }
-                    *reinterpret_cast<float4 *>(crow + 4 * q) = o;
+                    *reinterpret_cast<float4 *>(crow + 4 * j) = o;
                 }
             }
         }
     } else {
         // ------------------------------------------------------------ MMA issuer
-        constexpr uint32_t idesc = make_idesc(BM, BN, NEG, !NT && B_MN);
+        constexpr uint32_t idesc = make_idesc(BM, BN, NEG, false);
         for (int kb = 0; kb < nk; kb++) {
             const int s = kb % STAGES;
             mbar_wait(&full[s], (kb / STAGES) & 1);
             tc_fence_after();
             if (lane == 0) {
-                uint8_t *st = smem + s * S::STAGE;
-                const uint32_t a_big = smem_u32(st), a_small = a_big + S::A_BYTES;
-                const uint32_t b_big = a_big + 2 * S::A_BYTES, b_small = b_big + S::B_BYTES;
-                const bool bmn = !NT && B_MN;
+                uint8_t *st = smem + s * G::STAGE;
+                const uint32_t a_big = smem_u32(st), a_small = a_big + G::A_BYTES;
+                const uint32_t b_big = a_big + 2 * G::A_BYTES, b_small = b_big + G::B_BYTES;
 #pragma unroll
                 for (int kk = 0; kk < BK / 8; kk++) {
-                    // K-major: advance 32 B inside the 128 B swizzled row; MN-major: next k-group
-                    constexpr int var = VSK_MN_VARIANT;
-                    constexpr uint32_t s_atom = (var & 2) ? 1024 : 4096, s_kgrp = (var & 2) ? 4096 : 1024;
-                    const uint32_t ao = kk * 32, bo = bmn ? kk * s_kgrp : kk * 32;
-                    const uint32_t lbo = bmn ? ((var & 1) ? s_kgrp : s_atom) : 16;
-                    const uint32_t sbo = bmn ? ((var & 1) ? s_atom : s_kgrp) : 1024;
-                    const uint64_t dAb = make_desc(a_big + ao, 16, 1024), dAs = make_desc(a_small + ao, 16, 1024);
-                    const uint64_t dBb = make_desc(b_big + bo, lbo, sbo), dBs = make_desc(b_small + bo, lbo, sbo);
+                    // K-major SW128: the k-step advances 32 B inside the 128 B swizzled row
+                    const uint32_t o = kk * 32;
+                    const uint64_t dAb = make_desc(a_big + o, 16, 1024), dAs = make_desc(a_small + o, 16, 1024);
+                    const uint64_t dBb = make_desc(b_big + o, 16, 1024), dBs = make_desc(b_small + o, 16, 1024);
                     const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
                     mma_tf32(tmem, dAb, dBb, idesc, first);
                     mma_tf32(tmem, dAb, dBs, idesc, 1u);
@@ -316,24 +321,21 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
 
     tc_fence_before();
     __syncthreads();
-    if (warp == 4) {
+    if (warp == NPROD / 32) {
         tc_fence_after();
         asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)BN));
     }
 }
 
-// B_MN: NN operand B stored MN-major (vector STS) instead of transposed into K-major.
-// The MN-major descriptor path produced a zero contribution on the first B200 run, so the
-// transposing K-major path is the default until the MN-major encoding is probed.
-template <bool NT, bool NEG, bool LOWER, bool B_MN = false>
+// Host launcher: K multiple of 32; lda/ldb/ldc multiples of 4 and 16-byte aligned bases.
+template <bool NT, bool NEG, bool LOWER, int BN = 256>
 inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B, int ldb, float *C, int ldc,
                    cudaStream_t s)
 {
-    constexpr int BN = 128;
     if (M <= 0 || N <= 0) return 0;
     if (K % BK) return -1;
-    auto kern = tc_gemm_kernel<BN, NT, NEG, LOWER, B_MN>;
-    constexpr int smem = Smem<BN>::TOTAL;
+    auto kern = tc_gemm_kernel<BN, NT, NEG, LOWER>;
+    constexpr int smem = Cfg<BN>::SMEM;
     static bool attr[64] = {};
     int dev = 0;
     cudaGetDevice(&dev);
@@ -348,5 +350,4 @@ inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B,
 }
 
 }  // namespace tc
-
 }  // namespace vsk
