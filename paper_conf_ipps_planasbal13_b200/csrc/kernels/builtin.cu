@@ -1,17 +1,23 @@
 // builtin.cu — the built-in tile task versions (VS_T_* x VS_V_*): each version is a
 // sequence of sm_100a kernels enqueued on the worker's stream.
 //
-//   version        storage  GEMM engine (matmul/gemm/syrk + potrf/trsm updates)   panels
-//   simt_f32       fp32     simt_gemm<float,float>   (FFMA, bit-exact Fig 1 order)  fp32
-//   tc_3xtf32      fp32     tc_gemm (tcgen05/TMEM 3xTF32)                          fp32
-//   f64in_f32io    fp32     dmma_gemm<float>  (DMMA on upcast operands)            fp64
-//   dfma_f64       fp64     simt_gemm<double,double> (DFMA)                        fp64
-//   dmma_f64       fp64     dmma_gemm<double>  (mma.sync f64)                      fp64
+//   version        storage  GEMM engine (matmul/gemm/syrk + potrf/trsm updates)   trsm
+//   simt_f32       fp32     simt_gemm<float,float>   (FFMA, bit-exact Fig 1 order)  blocked
+//   tc_3xtf32      fp32     tc_gemm (tcgen05/TMEM 3xTF32)                          tc_trsm (1 launch)
+//   f64in_f32io    fp32     dmma_gemm<float>  (DMMA on upcast operands)            blocked
+//   dfma_f64       fp64     simt_gemm<double,double> (DFMA)                        blocked
+//   dmma_f64       fp64     dmma_gemm<double>  (mma.sync f64)                      blocked
+//
+// potrf (all versions) is recursive: potrf(A11); A21 <- A21 L11^{-T} (trsm);
+// A22 -= A21 A21^T (lower GEMM); potrf(A22), down to an NB x NB diagonal block factored
+// in shared memory (simt_chol.cuh).  Blocked trsm: NB-wide panels solved by trsm_panel,
+// remaining columns updated by the engine's GEMM.
 #include "dmma_gemm.cuh"
 #include "kernels.hpp"
 #include "simt_chol.cuh"
 #include "simt_gemm.cuh"
 #include "tc_gemm.cuh"
+#include "tc_trsm.cuh"
 
 #include "vsched.h"
 
@@ -19,38 +25,90 @@ namespace vsk {
 
 namespace {
 
+template <typename Tin, typename Tp, class Gemm>
+int blocked_trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s)
+{
+    constexpr int NBP = sizeof(Tp) == 4 ? 64 : 32;
+    for (int j0 = 0; j0 < n; j0 += NBP) {
+        trsm_panel<Tin, Tp, NBP>(L + (int64_t)j0 * ldl + j0, ldl, X + j0, ldx, rows, s);
+        const int rest = n - j0 - NBP;
+        if (rest > 0) {
+            int r = Gemm::template gemm<true, true, false>(rows, rest, NBP, X + j0, ldx, L + (int64_t)(j0 + NBP) * ldl + j0,
+                                                           ldl, X + j0 + NBP, ldx, s);
+            if (r) return r;
+        }
+    }
+    return 0;
+}
+
 template <typename Tin, typename Tacc>
 struct SimtEngine {
+    using Tp = Tacc;
     template <bool NT, bool NEG, bool LOWER>
     static int gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc, cudaStream_t s)
     {
         simt_gemm<Tin, Tacc, NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s);
         return 0;
     }
+    static int trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s)
+    {
+        return blocked_trsm<Tin, Tp, SimtEngine>(rows, n, L, ldl, X, ldx, s);
+    }
 };
 template <typename Tin>
 struct DmmaEngine {
+    using Tp = double;
     template <bool NT, bool NEG, bool LOWER>
     static int gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc, cudaStream_t s)
     {
         dmma_gemm<Tin, NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s);
         return 0;
     }
+    static int trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s)
+    {
+        return blocked_trsm<Tin, Tp, DmmaEngine>(rows, n, L, ldl, X, ldx, s);
+    }
 };
 struct TcEngine {
+    using Tp = float;
     template <bool NT, bool NEG, bool LOWER>
     static int gemm(int M, int N, int K, const float *A, int lda, const float *B, int ldb, float *C, int ldc,
                     cudaStream_t s)
     {
         return tc::tc_gemm<NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s);
     }
+    static int trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s)
+    {
+        return tc::tc_trsm(rows, n, L, ldl, X, ldx, s);
+    }
 };
 
-// Tin = storage, Tp = panel arithmetic, E = GEMM engine.
-template <typename Tin, typename Tp, class E>
+// Recursive Cholesky of the n x n lower block at A (leading dimension ld), global column
+// offset k_base (for info).
+template <typename Tin, class E>
+int potrf_rec(Tin *A, int n, int ld, int k_base, int *info, cudaStream_t s)
+{
+    using Tp = typename E::Tp;
+    constexpr int NBP = sizeof(Tp) == 4 ? 64 : 32;
+    if (n <= NBP) {
+        potrf_diag<Tin, Tp, NBP>(A, ld, k_base, info, s);
+        return 0;
+    }
+    int h = (n / 2) / 64 * 64;
+    if (h < NBP) h = NBP;
+    const int r = n - h;
+    Tin *A21 = A + (int64_t)h * ld, *A22 = A + (int64_t)h * ld + h;
+    int rc = potrf_rec<Tin, E>(A, h, ld, k_base, info, s);
+    if (!rc) rc = E::trsm(r, h, A, ld, A21, ld, s);
+    if (!rc) rc = E::template gemm<true, true, true>(r, r, h, A21, ld, A21, ld, A22, ld, s);
+    if (!rc) rc = potrf_rec<Tin, E>(A22, r, ld, k_base + h, info, s);
+    return rc;
+}
+
+// Tin = storage, E = engine.
+template <typename Tin, class E>
 int run_family(int type, int b, void *const *p, int *info, cudaStream_t s)
 {
-    constexpr int NBP = sizeof(Tp) == 4 ? 64 : 32;  // panel width (smem budget)
     switch (type) {
     case VS_T_MATMUL:  // C += A B                 (Fig 1)
         return E::template gemm<false, false, false>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[1], b, (Tin *)p[2], b, s);
@@ -58,35 +116,10 @@ int run_family(int type, int b, void *const *p, int *info, cudaStream_t s)
         return E::template gemm<true, true, false>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[1], b, (Tin *)p[2], b, s);
     case VS_T_SYRK:  // C -= A A^T, lower          (R5, R7)
         return E::template gemm<true, true, true>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[0], b, (Tin *)p[1], b, s);
-    case VS_T_TRSM: {  // B <- B L^{-T}            (R5)
-        const Tin *L = (const Tin *)p[0];
-        Tin *X = (Tin *)p[1];
-        for (int j0 = 0; j0 < b; j0 += NBP) {
-            trsm_panel<Tin, Tp, NBP>(L + (int64_t)j0 * b + j0, b, X + j0, b, b, s);
-            const int rest = b - j0 - NBP;
-            if (rest > 0) {
-                int r = E::template gemm<true, true, false>(b, rest, NBP, X + j0, b, L + (int64_t)(j0 + NBP) * b + j0, b,
-                                                            X + j0 + NBP, b, s);
-                if (r) return r;
-            }
-        }
-        return 0;
-    }
-    case VS_T_POTRF: {  // A = L L^T in place      (L697-699, R9)
-        Tin *A = (Tin *)p[0];
-        for (int k0 = 0; k0 < b; k0 += NBP) {
-            potrf_diag<Tin, Tp, NBP>(A + (int64_t)k0 * b + k0, b, k0, info, s);
-            const int rest = b - k0 - NBP;
-            if (rest > 0) {
-                trsm_panel<Tin, Tp, NBP>(A + (int64_t)k0 * b + k0, b, A + (int64_t)(k0 + NBP) * b + k0, b, rest, s);
-                Tin *P = A + (int64_t)(k0 + NBP) * b + k0;
-                int r = E::template gemm<true, true, true>(rest, rest, NBP, P, b, P, b, A + (int64_t)(k0 + NBP) * b + k0 + NBP,
-                                                           b, s);
-                if (r) return r;
-            }
-        }
-        return 0;
-    }
+    case VS_T_TRSM:  // B <- B L^{-T}              (R5)
+        return E::trsm(b, b, (const Tin *)p[0], b, (Tin *)p[1], b, s);
+    case VS_T_POTRF:  // A = L L^T in place        (L697-699, R9)
+        return potrf_rec<Tin, E>((Tin *)p[0], b, b, 0, info, s);
     }
     return -1;
 }
@@ -107,11 +140,11 @@ int launch_builtin(int type, int version, int b, void *const *p, int *info, cuda
 {
     if (!builtin_supported(type, version, b)) return -1;
     switch (version) {
-    case VS_V_SIMT_F32: return run_family<float, float, SimtEngine<float, float>>(type, b, p, info, s);
-    case VS_V_TC_3XTF32: return run_family<float, float, TcEngine>(type, b, p, info, s);
-    case VS_V_F64IN_F32IO: return run_family<float, double, DmmaEngine<float>>(type, b, p, info, s);
-    case VS_V_DFMA_F64: return run_family<double, double, SimtEngine<double, double>>(type, b, p, info, s);
-    case VS_V_DMMA_F64: return run_family<double, double, DmmaEngine<double>>(type, b, p, info, s);
+    case VS_V_SIMT_F32: return run_family<float, SimtEngine<float, float>>(type, b, p, info, s);
+    case VS_V_TC_3XTF32: return run_family<float, TcEngine>(type, b, p, info, s);
+    case VS_V_F64IN_F32IO: return run_family<float, DmmaEngine<float>>(type, b, p, info, s);
+    case VS_V_DFMA_F64: return run_family<double, SimtEngine<double, double>>(type, b, p, info, s);
+    case VS_V_DMMA_F64: return run_family<double, DmmaEngine<double>>(type, b, p, info, s);
     }
     return -1;
 }

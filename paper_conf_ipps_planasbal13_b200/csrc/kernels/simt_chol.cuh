@@ -1,14 +1,15 @@
 // simt_chol.cuh — SIMT building blocks of the potrf and trsm tile tasks (reading R5).
 //
-// potrf (in place, lower):  A = L L^T.  Blocked right-looking:
-//   for each nb-wide panel k0:  (1) potrf_diag: unblocked factorisation of the nb x nb
-//   diagonal block in shared memory (IEEE sqrt / div), first non-positive pivot ->
-//   *info (1-based, within the tile; R9);  (2) trsm_panel on the rows below;
-//   (3) lower-only NT GEMM update of the trailing matrix (simt_gemm / tc kernels).
-// trsm (right, lower, transposed, non-unit):  X L^T = B, X overwrites B.  Rows are
-//   independent; column panels J: (1) trsm_panel: per-row forward substitution
-//   x_j = (b_j - sum_{k<j} x_k L_jk) / L_jj  with L_JJ in shared memory; (2) NT GEMM
-//   update of the remaining columns.
+// potrf_diag: unblocked right-looking Cholesky of an NB x NB
+//   diagonal block, one CTA of NB threads; thread i keeps row i of the block in
+//   registers; per column k: thread k publishes l_kk = sqrt(a_kk) (first non-positive
+//   pivot -> *info, 1-based within the tile, R9), every thread i > k scales
+//   l_ik = a_ik / l_kk and publishes it, then updates its row a_ij -= l_ik l_jk
+//   (k < j <= i) from the published column: one barrier per column, IEEE sqrt/div.
+// trsm_panel: X <- X L^{-T} for an NB-wide column panel (right, lower, transposed,
+//   non-unit): each thread owns one row, forward substitution
+//   x_j = (b_j - sum_{k<j} x_k L_jk) / L_jj with L_JJ staged in shared memory.
+// Both stage their global tiles with fully unrolled, batched loads.
 #pragma once
 #include <cuda_runtime.h>
 #include <stdint.h>
@@ -17,48 +18,46 @@
 
 namespace vsk {
 
-// Unblocked right-looking Cholesky of an NB x NB diagonal block at A (leading dim lda),
-// computed in Tacc, lower triangle only.  One CTA.  k_base = global column of the block
-// (for info).  Writes back only j <= i.
 template <typename Tin, typename Tacc, int NB>
-__global__ void __launch_bounds__(256) potrf_diag_kernel(Tin *A, int lda, int k_base, int *info)
+__global__ void __launch_bounds__(NB) potrf_diag_kernel(Tin *A, int lda, int k_base, int *info)
 {
-    __shared__ Tacc a[NB][NB + 1];
+    __shared__ Tacc col[2][NB];   // published column k (double-buffered by parity)
     __shared__ int bad;
-    const int tid = threadIdx.x;
-    for (int e = tid; e < NB * NB; e += blockDim.x) {
-        const int i = e / NB, j = e % NB;
-        a[i][j] = j <= i ? (Tacc)A[(int64_t)i * lda + j] : (Tacc)0;
-    }
-    if (tid == 0) bad = 0;
+    const int i = threadIdx.x;
+    Tacc a[NB];
+    // row i, lower part only (j <= i); batched loads
+#pragma unroll
+    for (int j = 0; j < NB; j++) a[j] = (j <= i) ? (Tacc)A[(int64_t)i * lda + j] : (Tacc)0;
+    if (i == 0) bad = 0;
     __syncthreads();
+#pragma unroll
     for (int k = 0; k < NB; k++) {
-        if (tid == 0) {
-            const Tacc d = a[k][k];
-            if (!(d > (Tacc)0)) {
-                if (!bad) {
-                    bad = 1;
-                    if (info) atomicCAS(info, 0, k_base + k + 1);
-                }
+        if (i == k) {
+            const Tacc d = a[k];
+            if (!(d > (Tacc)0) && !bad) {
+                bad = 1;
+                if (info) atomicCAS(info, 0, k_base + k + 1);
             }
-            a[k][k] = sqrt(d);
+            a[k] = sqrt(d);
+            col[k & 1][k] = a[k];
         }
         __syncthreads();
-        const Tacc lkk = a[k][k];
-        for (int i = k + 1 + tid; i < NB; i += blockDim.x) a[i][k] = a[i][k] / lkk;
-        __syncthreads();
-        // trailing update a_ij -= a_ik * a_jk, k < j <= i
-        const int rem = NB - k - 1;
-        for (int e = tid; e < rem * rem; e += blockDim.x) {
-            const int i = k + 1 + e / rem, j = k + 1 + e % rem;
-            if (j <= i) a[i][j] = fma(-a[i][k], a[j][k], a[i][j]);
+        const Tacc lkk = col[k & 1][k];
+        if (i > k) {
+            a[k] = a[k] / lkk;
+            col[k & 1][i] = a[k];
         }
         __syncthreads();
+        if (i > k) {
+#pragma unroll
+            for (int j = k + 1; j < NB; j++)
+                if (j <= i) a[j] = fma(-a[k], col[k & 1][j], a[j]);
+        }
+        // buffer k&1 is rewritten at k+2, after every thread passed iteration k+1's barriers
     }
-    for (int e = tid; e < NB * NB; e += blockDim.x) {
-        const int i = e / NB, j = e % NB;
-        if (j <= i) A[(int64_t)i * lda + j] = (Tin)a[i][j];
-    }
+#pragma unroll
+    for (int j = 0; j < NB; j++)
+        if (j <= i) A[(int64_t)i * lda + j] = (Tin)a[j];
 }
 
 // Forward substitution of `rows` rows of X (leading dim ldx) against the NB x NB lower
@@ -70,13 +69,27 @@ __global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, T
     __shared__ Tacc x[64][NB + 1];
     const int tid = threadIdx.x;
     const int r0 = blockIdx.x * 64;
-    for (int e = tid; e < NB * NB; e += 64) {
-        const int i = e / NB, j = e % NB;
-        l[i][j] = j <= i ? (Tacc)L[(int64_t)i * ldl + j] : (Tacc)0;
+    constexpr int PER = NB * NB / 64;
+    Tin tmp[PER];
+#pragma unroll
+    for (int q = 0; q < PER; q++) {
+        const int e = tid + 64 * q, i = e / NB, j = e % NB;
+        tmp[q] = j <= i ? L[(int64_t)i * ldl + j] : (Tin)0;
     }
-    for (int e = tid; e < 64 * NB; e += 64) {
-        const int i = e / NB, j = e % NB;
-        x[i][j] = (r0 + i < rows) ? (Tacc)X[(int64_t)(r0 + i) * ldx + j] : (Tacc)0;
+#pragma unroll
+    for (int q = 0; q < PER; q++) {
+        const int e = tid + 64 * q, i = e / NB, j = e % NB;
+        l[i][j] = (Tacc)tmp[q];
+    }
+#pragma unroll
+    for (int q = 0; q < PER; q++) {
+        const int e = tid + 64 * q, i = e / NB, j = e % NB;
+        tmp[q] = (r0 + i < rows) ? X[(int64_t)(r0 + i) * ldx + j] : (Tin)0;
+    }
+#pragma unroll
+    for (int q = 0; q < PER; q++) {
+        const int e = tid + 64 * q, i = e / NB, j = e % NB;
+        x[i][j] = (Tacc)tmp[q];
     }
     __syncthreads();
     for (int j = 0; j < NB; j++) {
@@ -85,8 +98,9 @@ __global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, T
         x[tid][j] = s / l[j][j];
     }
     __syncthreads();
-    for (int e = tid; e < 64 * NB; e += 64) {
-        const int i = e / NB, j = e % NB;
+#pragma unroll
+    for (int q = 0; q < PER; q++) {
+        const int e = tid + 64 * q, i = e / NB, j = e % NB;
         if (r0 + i < rows) X[(int64_t)(r0 + i) * ldx + j] = (Tin)x[i][j];
     }
 }
@@ -95,7 +109,7 @@ template <typename Tin, typename Tacc, int NB>
 inline void potrf_diag(Tin *A, int lda, int k_base, int *info, cudaStream_t s)
 {
     count_launch();
-    potrf_diag_kernel<Tin, Tacc, NB><<<1, 256, 0, s>>>(A, lda, k_base, info);
+    potrf_diag_kernel<Tin, Tacc, NB><<<1, NB, 0, s>>>(A, lda, k_base, info);
 }
 
 template <typename Tin, typename Tacc, int NB>
