@@ -81,15 +81,17 @@ __global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, T
         const int e = tid + 64 * q, i = e / NB, j = e % NB;
         l[i][j] = (Tacc)tmp[q];
     }
+    constexpr int PERX = NB;   // 64 rows x NB columns over 64 threads
+    Tin tmx[PERX];
 #pragma unroll
-    for (int q = 0; q < PER; q++) {
+    for (int q = 0; q < PERX; q++) {
         const int e = tid + 64 * q, i = e / NB, j = e % NB;
-        tmp[q] = (r0 + i < rows) ? X[(int64_t)(r0 + i) * ldx + j] : (Tin)0;
+        tmx[q] = (r0 + i < rows) ? X[(int64_t)(r0 + i) * ldx + j] : (Tin)0;
     }
 #pragma unroll
-    for (int q = 0; q < PER; q++) {
+    for (int q = 0; q < PERX; q++) {
         const int e = tid + 64 * q, i = e / NB, j = e % NB;
-        x[i][j] = (Tacc)tmp[q];
+        x[i][j] = (Tacc)tmx[q];
     }
     __syncthreads();
     for (int j = 0; j < NB; j++) {
@@ -99,7 +101,7 @@ __global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, T
     }
     __syncthreads();
 #pragma unroll
-    for (int q = 0; q < PER; q++) {
+    for (int q = 0; q < PERX; q++) {
         const int e = tid + 64 * q, i = e / NB, j = e % NB;
         if (r0 + i < rows) X[(int64_t)(r0 + i) * ldx + j] = (Tin)x[i][j];
     }

@@ -104,6 +104,18 @@ __device__ __forceinline__ void mma_commit(uint64_t *bar)
                  : "memory");
 }
 
+__device__ __forceinline__ void tmem_st32(uint32_t taddr, const float (&v)[32])
+{
+    asm volatile(
+        "tcgen05.st.sync.aligned.32x32b.x32.b32 [%0], {%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,%16,"
+        "%17,%18,%19,%20,%21,%22,%23,%24,%25,%26,%27,%28,%29,%30,%31,%32};" ::"r"(taddr),
+        "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(v[4]), "f"(v[5]), "f"(v[6]), "f"(v[7]), "f"(v[8]), "f"(v[9]),
+        "f"(v[10]), "f"(v[11]), "f"(v[12]), "f"(v[13]), "f"(v[14]), "f"(v[15]), "f"(v[16]), "f"(v[17]), "f"(v[18]),
+        "f"(v[19]), "f"(v[20]), "f"(v[21]), "f"(v[22]), "f"(v[23]), "f"(v[24]), "f"(v[25]), "f"(v[26]), "f"(v[27]),
+        "f"(v[28]), "f"(v[29]), "f"(v[30]), "f"(v[31])
+        : "memory");
+}
+
 __device__ __forceinline__ void tmem_ld32(uint32_t taddr, float (&v)[32])
 {
     uint32_t r[32];
@@ -161,7 +173,8 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     uint64_t *full = (uint64_t *)(smem + STAGES * G::STAGE);
     uint64_t *empty = full + STAGES;
     uint64_t *acc_full = empty + STAGES;
-    uint32_t *tmem_slot = (uint32_t *)(acc_full + 1);
+    uint64_t *c_ready = acc_full + 1;
+    uint32_t *tmem_slot = (uint32_t *)(c_ready + 1);
 
     const int m0 = blockIdx.y * BM, n0 = blockIdx.x * BN;
     if (LOWER && n0 >= m0 + BM) return;
@@ -174,6 +187,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
             mbar_init(&empty[s], 1);
         }
         mbar_init(acc_full, 1);
+        mbar_init(c_ready, NPROD);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     }
     if (warp == NPROD / 32) {
@@ -239,10 +253,18 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                     const int u = t + p * NPROD, kq = u / (BN / 4), nq = u % (BN / 4);
                     const float4 r0 = rb[4 * p], r1 = rb[4 * p + 1], r2 = rb[4 * p + 2], r3 = rb[4 * p + 3];
                     // column n' of the 4x4 block = K-major 16-byte chunk of row n = 4nq+n'
-                    store_split(b_big, b_small, kmaj_off(4 * nq + 0, kq), make_float4(r0.x, r1.x, r2.x, r3.x));
-                    store_split(b_big, b_small, kmaj_off(4 * nq + 1, kq), make_float4(r0.y, r1.y, r2.y, r3.y));
-                    store_split(b_big, b_small, kmaj_off(4 * nq + 2, kq), make_float4(r0.z, r1.z, r2.z, r3.z));
-                    store_split(b_big, b_small, kmaj_off(4 * nq + 3, kq), make_float4(r0.w, r1.w, r2.w, r3.w));
+                    // rotate which column each thread stores first so the 8 threads of an
+                    // STS.128 phase hit 8 distinct (row & 7) -> 8 distinct swizzled chunks
+                    const int rot = (nq >> 1) & 3;
+#pragma unroll
+                    for (int qq = 0; qq < 4; qq++) {
+                        const int i = (qq + rot) & 3;
+                        const float4 col = i == 0 ? make_float4(r0.x, r1.x, r2.x, r3.x)
+                                         : i == 1 ? make_float4(r0.y, r1.y, r2.y, r3.y)
+                                         : i == 2 ? make_float4(r0.z, r1.z, r2.z, r3.z)
+                                                  : make_float4(r0.w, r1.w, r2.w, r3.w);
+                        store_split(b_big, b_small, kmaj_off(4 * nq + i, kq), col);
+                    }
                 }
             }
             fence_proxy_async();
@@ -252,6 +274,25 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
         float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
         load(ra0, rb0, 0);
         if (nk > 1) load(ra1, rb1, 1);
+        // preload the C tile into the TMEM accumulator (this warp: lane quarter eq, column
+        // half eh) while the first k-blocks are in flight; the MMAs then accumulate onto it
+        const int eq = warp & 3, eh = warp >> 2;
+        const int erow = m0 + eq * 32 + lane;
+#pragma unroll 1
+        for (int c = 0; c < BN / 64; c++) {
+            const int col0 = eh * (BN / 2) + c * 32;
+            float v[32];
+            const float *crow = C + (int64_t)erow * ldc + n0 + col0;
+#pragma unroll
+            for (int j = 0; j < 8; j++) {
+                const float4 x = (erow < M && n0 + col0 + 4 * j < N) ? *reinterpret_cast<const float4 *>(crow + 4 * j) : z4;
+                v[4 * j] = x.x; v[4 * j + 1] = x.y; v[4 * j + 2] = x.z; v[4 * j + 3] = x.w;
+            }
+            tmem_st32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)col0, v);
+        }
+        asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
+        tc_fence_before();
+        mbar_arrive(c_ready);
         for (int kb = 0; kb < nk; kb += 2) {
             produce(ra0, rb0, kb);
             if (kb + 2 < nk) load(ra0, rb0, kb + 2);
@@ -264,29 +305,26 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
         // ------------------------------------------------------------ epilogue
         mbar_wait(acc_full, 0);
         tc_fence_after();
-        const int q = warp & 3, h = warp >> 2;
-        const int row = m0 + q * 32 + lane;
+        // C was preloaded into the accumulator: store-only epilogue
 #pragma unroll 1
         for (int c = 0; c < BN / 64; c++) {
-            const int col0 = h * (BN / 2) + c * 32;
+            const int col0 = eh * (BN / 2) + c * 32;
             float v[32];
-            tmem_ld32(tmem + ((uint32_t)(q * 32) << 16) + (uint32_t)col0, v);
-            if (row < M) {
-                float *crow = C + (int64_t)row * ldc + n0 + col0;
+            tmem_ld32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)col0, v);
+            if (erow < M) {
+                float *crow = C + (int64_t)erow * ldc + n0 + col0;
 #pragma unroll
                 for (int j = 0; j < 8; j++) {
                     const int col = n0 + col0 + 4 * j;
                     if (col >= N) break;
-                    float4 o = *reinterpret_cast<float4 *>(crow + 4 * j);
-                    if (LOWER && col + 3 > row) {
-                        if (col + 0 <= row) o.x += v[4 * j + 0];
-                        if (col + 1 <= row) o.y += v[4 * j + 1];
-                        if (col + 2 <= row) o.z += v[4 * j + 2];
-                        if (col + 3 <= row) o.w += v[4 * j + 3];
+                    if (LOWER && col + 3 > erow) {
+                        if (col + 0 <= erow) crow[4 * j + 0] = v[4 * j + 0];
+                        if (col + 1 <= erow) crow[4 * j + 1] = v[4 * j + 1];
+                        if (col + 2 <= erow) crow[4 * j + 2] = v[4 * j + 2];
                     } else {
-                        o.x += v[4 * j + 0]; o.y += v[4 * j + 1]; o.z += v[4 * j + 2]; o.w += v[4 * j + 3];
+                        *reinterpret_cast<float4 *>(crow + 4 * j) =
+                            make_float4(v[4 * j + 0], v[4 * j + 1], v[4 * j + 2], v[4 * j + 3]);
                     }
-                    *reinterpret_cast<float4 *>(crow + 4 * j) = o;
                 }
             }
         }
@@ -295,6 +333,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
         constexpr uint32_t idesc = make_idesc(BM, BN, NEG, false);
         for (int kb = 0; kb < nk; kb++) {
             const int s = kb % STAGES;
+            if (kb == 0) mbar_wait(c_ready, 0);
             mbar_wait(&full[s], (kb / STAGES) & 1);
             tc_fence_after();
             if (lane == 0) {
@@ -307,8 +346,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                     const uint32_t o = kk * 32;
                     const uint64_t dAb = make_desc(a_big + o, 16, 1024), dAs = make_desc(a_small + o, 16, 1024);
                     const uint64_t dBb = make_desc(b_big + o, 16, 1024), dBs = make_desc(b_small + o, 16, 1024);
-                    const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
-                    mma_tf32(tmem, dAb, dBb, idesc, first);
+                    mma_tf32(tmem, dAb, dBb, idesc, 1u);   // accumulate onto the preloaded C
                     mma_tf32(tmem, dAb, dBs, idesc, 1u);
                     mma_tf32(tmem, dAs, dBb, idesc, 1u);
                 }

@@ -33,6 +33,22 @@ struct TrsmCfg {
     static constexpr int BPER = TRSM_P * BK / 4 / NPROD;  // 2
 };
 
+__device__ __forceinline__ float rcp_approx(float x)
+{
+    float r;
+    asm("rcp.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(x));
+    return r;
+}
+// t / l without the IEEE-division slow-path call (which forces the per-thread row into
+// local memory): x0 = t r, one Newton correction x = x0 + (t - x0 l) r.  For a positive
+// normal l this is the correctly rounded quotient whenever t / l is representable
+// (integer problems stay exact) and within 1 ulp otherwise.
+__device__ __forceinline__ float div_nr(float t, float l, float r)
+{
+    const float x0 = t * r;
+    return fmaf(fmaf(-x0, l, t), r, x0);
+}
+
 __device__ __forceinline__ float4 ld_f4_coherent(const float *p)
 {
     float4 v;
@@ -48,6 +64,7 @@ tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, 
     extern __shared__ uint8_t smem_raw[];
     uint8_t *smem = (uint8_t *)(((uintptr_t)smem_raw + 1023) & ~(uintptr_t)1023);
     float(*Ls)[P + 1] = reinterpret_cast<float(*)[P + 1]>(smem + STAGES * G::STAGE);
+    __shared__ float Lr[P];   // approximate reciprocals of the diagonal of L_JJ
     uint64_t *full = (uint64_t *)(smem + STAGES * G::STAGE + G::LS_BYTES);
     uint64_t *empty = full + STAGES;
     uint64_t *acc_full = empty + STAGES;
@@ -95,6 +112,7 @@ tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, 
                     const int e = t + q * NPROD, i = e / P, j = e % P;
                     Ls[i][j] = tmp[q];
                 }
+                if (t < P) Lr[t] = rcp_approx(__ldg(L + (int64_t)(c0 + t) * ldl + c0 + t));
             }
             // ---- producers: A = X[m0.., 0:c0] (coherent loads), B = L[c0..c0+P, 0:c0] (K-major)
             constexpr int APER = G::APER, BPER = G::BPER;
@@ -173,9 +191,10 @@ tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, 
                     }
 #pragma unroll
                     for (int c = 0; c < P; c++) {
-                        tv[c] = tv[c] / Ls[c][c];
+                        tv[c] = div_nr(tv[c], Ls[c][c], Lr[c]);
 #pragma unroll
-                        for (int j = c + 1; j < P; j++) tv[j] = fmaf(-tv[c], Ls[j][c], tv[j]);
+                        for (int j = 0; j < P; j++)
+                            if (j > c) tv[j] = fmaf(-tv[c], Ls[j][c], tv[j]);
                     }
 #pragma unroll
                     for (int q = 0; q < P / 4; q++)
