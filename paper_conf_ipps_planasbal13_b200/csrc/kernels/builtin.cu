@@ -1,5 +1,7 @@
 // builtin.cu — the built-in tile task versions (VS_T_* x VS_V_*): each version is a
-// sequence of sm_100a kernels enqueued on the worker's stream.
+// sequence of sm_100a kernels enqueued on the worker's stream.  Every kernel receives the
+// task's TaskCtx (task_ctx.cuh) so the task's GPU execution interval is recorded on the
+// device.
 //
 //   version        storage  GEMM engine (matmul/gemm/syrk + potrf/trsm updates)   trsm
 //   simt_f32       fp32     simt_gemm<float,float>   (FFMA, bit-exact Fig 1 order)  blocked
@@ -10,7 +12,7 @@
 //
 // potrf (all versions) is recursive: potrf(A11); A21 <- A21 L11^{-T} (trsm);
 // A22 -= A21 A21^T (lower GEMM); potrf(A22), down to an NB x NB diagonal block factored
-// in shared memory (simt_chol.cuh).  Blocked trsm: NB-wide panels solved by trsm_panel,
+// in registers (simt_chol.cuh).  Blocked trsm: NB-wide panels solved by trsm_panel,
 // remaining columns updated by the engine's GEMM.
 #include "dmma_gemm.cuh"
 #include "kernels.hpp"
@@ -26,15 +28,15 @@ namespace vsk {
 namespace {
 
 template <typename Tin, typename Tp, class Gemm>
-int blocked_trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s)
+int blocked_trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
 {
     constexpr int NBP = sizeof(Tp) == 4 ? 64 : 32;
     for (int j0 = 0; j0 < n; j0 += NBP) {
-        trsm_panel<Tin, Tp, NBP>(L + (int64_t)j0 * ldl + j0, ldl, X + j0, ldx, rows, s);
+        trsm_panel<Tin, Tp, NBP>(L + (int64_t)j0 * ldl + j0, ldl, X + j0, ldx, rows, s, ctx);
         const int rest = n - j0 - NBP;
         if (rest > 0) {
             int r = Gemm::template gemm<true, true, false>(rows, rest, NBP, X + j0, ldx, L + (int64_t)(j0 + NBP) * ldl + j0,
-                                                           ldl, X + j0 + NBP, ldx, s);
+                                                           ldl, X + j0 + NBP, ldx, s, ctx);
             if (r) return r;
         }
     }
@@ -45,81 +47,86 @@ template <typename Tin, typename Tacc>
 struct SimtEngine {
     using Tp = Tacc;
     template <bool NT, bool NEG, bool LOWER>
-    static int gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc, cudaStream_t s)
+    static int gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc, cudaStream_t s,
+                    const TaskCtx &ctx)
     {
-        simt_gemm<Tin, Tacc, NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s);
+        simt_gemm<Tin, Tacc, NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s, ctx);
         return 0;
     }
-    static int trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s)
+    static int trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
     {
-        return blocked_trsm<Tin, Tp, SimtEngine>(rows, n, L, ldl, X, ldx, s);
+        return blocked_trsm<Tin, Tp, SimtEngine>(rows, n, L, ldl, X, ldx, s, ctx);
     }
 };
 template <typename Tin>
 struct DmmaEngine {
     using Tp = double;
     template <bool NT, bool NEG, bool LOWER>
-    static int gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc, cudaStream_t s)
+    static int gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc, cudaStream_t s,
+                    const TaskCtx &ctx)
     {
-        dmma_gemm<Tin, NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s);
+        dmma_gemm<Tin, NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s, ctx);
         return 0;
     }
-    static int trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s)
+    static int trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
     {
-        return blocked_trsm<Tin, Tp, DmmaEngine>(rows, n, L, ldl, X, ldx, s);
+        return blocked_trsm<Tin, Tp, DmmaEngine>(rows, n, L, ldl, X, ldx, s, ctx);
     }
 };
 struct TcEngine {
     using Tp = float;
     template <bool NT, bool NEG, bool LOWER>
     static int gemm(int M, int N, int K, const float *A, int lda, const float *B, int ldb, float *C, int ldc,
-                    cudaStream_t s)
+                    cudaStream_t s, const TaskCtx &ctx)
     {
-        return tc::tc_gemm<NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s);
+        return tc::tc_gemm<NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s, ctx);
     }
-    static int trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s)
+    static int trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
     {
-        return tc::tc_trsm(rows, n, L, ldl, X, ldx, s);
+        return tc::tc_trsm(rows, n, L, ldl, X, ldx, s, ctx);
     }
 };
 
 // Recursive Cholesky of the n x n lower block at A (leading dimension ld), global column
 // offset k_base (for info).
 template <typename Tin, class E>
-int potrf_rec(Tin *A, int n, int ld, int k_base, int *info, cudaStream_t s)
+int potrf_rec(Tin *A, int n, int ld, int k_base, int *info, cudaStream_t s, const TaskCtx &ctx)
 {
     using Tp = typename E::Tp;
     constexpr int NBP = sizeof(Tp) == 4 ? 64 : 32;
     if (n <= NBP) {
-        potrf_diag<Tin, Tp, NBP>(A, ld, k_base, info, s);
+        potrf_diag<Tin, Tp, NBP>(A, ld, k_base, info, s, ctx);
         return 0;
     }
     int h = (n / 2) / 64 * 64;
     if (h < NBP) h = NBP;
     const int r = n - h;
     Tin *A21 = A + (int64_t)h * ld, *A22 = A + (int64_t)h * ld + h;
-    int rc = potrf_rec<Tin, E>(A, h, ld, k_base, info, s);
-    if (!rc) rc = E::trsm(r, h, A, ld, A21, ld, s);
-    if (!rc) rc = E::template gemm<true, true, true>(r, r, h, A21, ld, A21, ld, A22, ld, s);
-    if (!rc) rc = potrf_rec<Tin, E>(A22, r, ld, k_base + h, info, s);
+    int rc = potrf_rec<Tin, E>(A, h, ld, k_base, info, s, ctx);
+    if (!rc) rc = E::trsm(r, h, A, ld, A21, ld, s, ctx);
+    if (!rc) rc = E::template gemm<true, true, true>(r, r, h, A21, ld, A21, ld, A22, ld, s, ctx);
+    if (!rc) rc = potrf_rec<Tin, E>(A22, r, ld, k_base + h, info, s, ctx);
     return rc;
 }
 
 // Tin = storage, E = engine.
 template <typename Tin, class E>
-int run_family(int type, int b, void *const *p, int *info, cudaStream_t s)
+int run_family(int type, int b, void *const *p, int *info, cudaStream_t s, const TaskCtx &ctx)
 {
     switch (type) {
     case VS_T_MATMUL:  // C += A B                 (Fig 1)
-        return E::template gemm<false, false, false>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[1], b, (Tin *)p[2], b, s);
+        return E::template gemm<false, false, false>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[1], b, (Tin *)p[2], b,
+                                                     s, ctx);
     case VS_T_GEMM_NT:  // C -= A B^T              (R5)
-        return E::template gemm<true, true, false>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[1], b, (Tin *)p[2], b, s);
+        return E::template gemm<true, true, false>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[1], b, (Tin *)p[2], b,
+                                                   s, ctx);
     case VS_T_SYRK:  // C -= A A^T, lower          (R5, R7)
-        return E::template gemm<true, true, true>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[0], b, (Tin *)p[1], b, s);
+        return E::template gemm<true, true, true>(b, b, b, (const Tin *)p[0], b, (const Tin *)p[0], b, (Tin *)p[1], b, s,
+                                                  ctx);
     case VS_T_TRSM:  // B <- B L^{-T}              (R5)
-        return E::trsm(b, b, (const Tin *)p[0], b, (Tin *)p[1], b, s);
+        return E::trsm(b, b, (const Tin *)p[0], b, (Tin *)p[1], b, s, ctx);
     case VS_T_POTRF:  // A = L L^T in place        (L697-699, R9)
-        return potrf_rec<Tin, E>((Tin *)p[0], b, b, 0, info, s);
+        return potrf_rec<Tin, E>((Tin *)p[0], b, b, 0, info, s, ctx);
     }
     return -1;
 }
@@ -136,15 +143,15 @@ bool builtin_supported(int type, int version, int b)
     return true;
 }
 
-int launch_builtin(int type, int version, int b, void *const *p, int *info, cudaStream_t s)
+int launch_builtin(int type, int version, int b, void *const *p, int *info, cudaStream_t s, const TaskCtx &ctx)
 {
     if (!builtin_supported(type, version, b)) return -1;
     switch (version) {
-    case VS_V_SIMT_F32: return run_family<float, SimtEngine<float, float>>(type, b, p, info, s);
-    case VS_V_TC_3XTF32: return run_family<float, TcEngine>(type, b, p, info, s);
-    case VS_V_F64IN_F32IO: return run_family<float, DmmaEngine<float>>(type, b, p, info, s);
-    case VS_V_DFMA_F64: return run_family<double, SimtEngine<double, double>>(type, b, p, info, s);
-    case VS_V_DMMA_F64: return run_family<double, DmmaEngine<double>>(type, b, p, info, s);
+    case VS_V_SIMT_F32: return run_family<float, SimtEngine<float, float>>(type, b, p, info, s, ctx);
+    case VS_V_TC_3XTF32: return run_family<float, TcEngine>(type, b, p, info, s, ctx);
+    case VS_V_F64IN_F32IO: return run_family<float, DmmaEngine<float>>(type, b, p, info, s, ctx);
+    case VS_V_DFMA_F64: return run_family<double, SimtEngine<double, double>>(type, b, p, info, s, ctx);
+    case VS_V_DMMA_F64: return run_family<double, DmmaEngine<double>>(type, b, p, info, s, ctx);
     }
     return -1;
 }

@@ -16,6 +16,7 @@
 #include <stdint.h>
 
 #include "kernels.hpp"
+#include "task_ctx.cuh"
 
 namespace vsk {
 
@@ -29,13 +30,17 @@ __device__ __forceinline__ void dmma_8x8x4(double &d0, double &d1, double a, dou
 template <typename Tin, bool NT, bool NEG, bool LOWER>
 __global__ void __launch_bounds__(128) dmma_gemm_kernel(int M, int N, int K, const Tin *__restrict__ A, int lda,
                                                         const Tin *__restrict__ B, int ldb, Tin *__restrict__ C,
-                                                        int ldc)
+                                                        int ldc, TaskCtx ctx)
 {
+    ctx_begin(ctx);
     constexpr int BM = 64, BN = 64, BK = 16;
     __shared__ double As[BM][BK + 1];
     __shared__ double Bs[BK][BN + 1];
     const int m0 = blockIdx.y * BM, n0 = blockIdx.x * BN;
-    if (LOWER && n0 >= m0 + BM) return;
+    if (LOWER && n0 >= m0 + BM) {
+        ctx_end(ctx);
+        return;
+    }
     const int tid = threadIdx.x, warp = tid >> 5, lane = tid & 31;
     const int wm = (warp >> 1) * 32, wn = (warp & 1) * 32;
     const int g = lane >> 2, t = lane & 3;
@@ -90,16 +95,17 @@ __global__ void __launch_bounds__(128) dmma_gemm_kernel(int M, int N, int K, con
                 const int r = m0 + wm + 8 * i + g, c = n0 + wn + 8 * j + 2 * t + e;
                 if (r < M && c < N && (!LOWER || c <= r)) C[(int64_t)r * ldc + c] = (Tin)acc[i][j][e];
             }
+    ctx_end(ctx);
 }
 
 template <typename Tin, bool NT, bool NEG, bool LOWER>
 inline void dmma_gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc,
-                      cudaStream_t s)
+                      cudaStream_t s, const TaskCtx &ctx)
 {
     if (M <= 0 || N <= 0) return;
     dim3 grid((N + 63) / 64, (M + 63) / 64);
     count_launch();
-    dmma_gemm_kernel<Tin, NT, NEG, LOWER><<<grid, 128, 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc);
+    dmma_gemm_kernel<Tin, NT, NEG, LOWER><<<grid, 128, 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc, ctx);
 }
 
 }  // namespace vsk

@@ -16,9 +16,18 @@ inline std::atomic<long long> &launch_counter()
 }
 inline void count_launch() { launch_counter().fetch_add(1, std::memory_order_relaxed); }
 
+// Per-task execution record passed to every kernel of a built-in version (task_ctx.cuh).
+// slot: device memory {start_min, end_max, ticket}; host: host-mapped {start, end}.
+// A default TaskCtx (nullptrs) disables recording (direct vs_tile_run calls).
+struct TaskCtx {
+    unsigned long long *slot = nullptr;
+    unsigned long long *host = nullptr;
+};
+
 // Task types / versions use the VS_T_* / VS_V_* numbering of vsched.h.
 // Returns 0 on success, -1 for an unsupported (type, version, b).
-int launch_builtin(int type, int version, int b, void *const *p, int *dinfo, cudaStream_t s);
+int launch_builtin(int type, int version, int b, void *const *p, int *dinfo, cudaStream_t s,
+                   const TaskCtx &ctx = TaskCtx());
 bool builtin_supported(int type, int version, int b);
 // Element size in bytes for a version (4 for f32-io versions, 8 for f64).
 int builtin_elem_bytes(int version);

@@ -15,12 +15,14 @@
 #include <stdint.h>
 
 #include "kernels.hpp"
+#include "task_ctx.cuh"
 
 namespace vsk {
 
 template <typename Tin, typename Tacc, int NB>
-__global__ void __launch_bounds__(NB) potrf_diag_kernel(Tin *A, int lda, int k_base, int *info)
+__global__ void __launch_bounds__(NB) potrf_diag_kernel(Tin *A, int lda, int k_base, int *info, TaskCtx ctx)
 {
+    ctx_begin(ctx);
     __shared__ Tacc col[2][NB];   // published column k (double-buffered by parity)
     __shared__ int bad;
     const int i = threadIdx.x;
@@ -58,13 +60,15 @@ __global__ void __launch_bounds__(NB) potrf_diag_kernel(Tin *A, int lda, int k_b
 #pragma unroll
     for (int j = 0; j < NB; j++)
         if (j <= i) A[(int64_t)i * lda + j] = (Tin)a[j];
+    ctx_end(ctx);
 }
 
 // Forward substitution of `rows` rows of X (leading dim ldx) against the NB x NB lower
 // block L (leading dim ldl):  X <- X L^{-T}.  Each CTA owns 64 rows staged in smem.
 template <typename Tin, typename Tacc, int NB>
-__global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, Tin *X, int ldx, int rows)
+__global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, Tin *X, int ldx, int rows, TaskCtx ctx)
 {
+    ctx_begin(ctx);
     __shared__ Tacc l[NB][NB + 1];
     __shared__ Tacc x[64][NB + 1];
     const int tid = threadIdx.x;
@@ -105,21 +109,22 @@ __global__ void __launch_bounds__(64) trsm_panel_kernel(const Tin *L, int ldl, T
         const int e = tid + 64 * q, i = e / NB, j = e % NB;
         if (r0 + i < rows) X[(int64_t)(r0 + i) * ldx + j] = (Tin)x[i][j];
     }
+    ctx_end(ctx);
 }
 
 template <typename Tin, typename Tacc, int NB>
-inline void potrf_diag(Tin *A, int lda, int k_base, int *info, cudaStream_t s)
+inline void potrf_diag(Tin *A, int lda, int k_base, int *info, cudaStream_t s, const TaskCtx &ctx)
 {
     count_launch();
-    potrf_diag_kernel<Tin, Tacc, NB><<<1, NB, 0, s>>>(A, lda, k_base, info);
+    potrf_diag_kernel<Tin, Tacc, NB><<<1, NB, 0, s>>>(A, lda, k_base, info, ctx);
 }
 
 template <typename Tin, typename Tacc, int NB>
-inline void trsm_panel(const Tin *L, int ldl, Tin *X, int ldx, int rows, cudaStream_t s)
+inline void trsm_panel(const Tin *L, int ldl, Tin *X, int ldx, int rows, cudaStream_t s, const TaskCtx &ctx)
 {
     if (rows <= 0) return;
     count_launch();
-    trsm_panel_kernel<Tin, Tacc, NB><<<(rows + 63) / 64, 64, 0, s>>>(L, ldl, X, ldx, rows);
+    trsm_panel_kernel<Tin, Tacc, NB><<<(rows + 63) / 64, 64, 0, s>>>(L, ldl, X, ldx, rows, ctx);
 }
 
 }  // namespace vsk

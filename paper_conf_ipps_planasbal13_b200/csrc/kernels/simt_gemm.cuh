@@ -20,6 +20,7 @@
 #include <stdint.h>
 
 #include "kernels.hpp"
+#include "task_ctx.cuh"
 
 namespace vsk {
 
@@ -30,8 +31,9 @@ template <> struct Vec16<double> { using type = double2; static constexpr int n 
 template <typename Tin, typename Tacc, int BM, int BN, int BK, int TM, int TN, bool NT, bool NEG, bool LOWER>
 __global__ void __launch_bounds__((BM / TM) * (BN / TN))
 simt_gemm_kernel(int M, int N, int K, const Tin *__restrict__ A, int lda, const Tin *__restrict__ B, int ldb,
-                 Tin *__restrict__ C, int ldc)
+                 Tin *__restrict__ C, int ldc, TaskCtx ctx)
 {
+    ctx_begin(ctx);
     constexpr int NTH = (BM / TM) * (BN / TN);
     using V = typename Vec16<Tin>::type;
     constexpr int VN = Vec16<Tin>::n;
@@ -45,7 +47,10 @@ simt_gemm_kernel(int M, int N, int K, const Tin *__restrict__ A, int lda, const 
     __shared__ __align__(16) Tacc Bs[BK][BN + 4];
 
     const int m0 = blockIdx.y * BM, n0 = blockIdx.x * BN;
-    if (LOWER && n0 >= m0 + BM) return;               // tile strictly above the diagonal
+    if (LOWER && n0 >= m0 + BM) {                     // tile strictly above the diagonal
+        ctx_end(ctx);
+        return;
+    }
     const int tid = threadIdx.x;
     const int tx = tid % (BN / TN), ty = tid / (BN / TN);
 
@@ -137,13 +142,14 @@ simt_gemm_kernel(int M, int N, int K, const Tin *__restrict__ A, int lda, const 
             const int r = m0 + ty * TM + i, c = n0 + tx * TN + j;
             if (r < M && c < N && (!LOWER || c <= r)) C[(int64_t)r * ldc + c] = (Tin)acc[i][j];
         }
+    ctx_end(ctx);
 }
 
 // Host launcher.  K must be a multiple of BK (16); lda/ldb and the k offsets must keep
 // 16-byte alignment (tile sizes are multiples of 32 elements).
 template <typename Tin, typename Tacc, bool NT, bool NEG, bool LOWER>
 inline void simt_gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, int ldb, Tin *C, int ldc,
-                      cudaStream_t s)
+                      cudaStream_t s, const TaskCtx &ctx)
 {
     if (M <= 0 || N <= 0) return;
     constexpr bool WIDE = sizeof(Tacc) == 4;           // fp32 math: 128x128 tiles, 8x8 per thread
@@ -151,7 +157,7 @@ inline void simt_gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, 
     dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
     count_launch();
     simt_gemm_kernel<Tin, Tacc, BM, BN, BK, TM, TN, NT, NEG, LOWER>
-        <<<grid, (BM / TM) * (BN / TN), 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc);
+        <<<grid, (BM / TM) * (BN / TN), 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc, ctx);
 }
 
 }  // namespace vsk

@@ -1,0 +1,56 @@
+// task_ctx.cuh — device-side execution-time record of one task (a14, reading R17).
+//
+// Every kernel of a built-in version receives the task's TaskCtx.  The first thread of
+// each CTA folds %globaltimer into the task's device slot when the CTA starts
+// (atomicMax of ~t, i.e. the minimum start) and ends (atomicMax); the last CTA of every
+// kernel (ticket) copies the current {~start, end} into the task's host-mapped slot and
+// re-arms the ticket.  Kernels
+// of one task run in stream order, so the host slot holds [first CTA start of the first
+// kernel, last CTA end of the last kernel] once the task's completion event has fired:
+// the time the task really occupied the GPU, without the time its launch waited in the
+// stream queue (which CUDA events would include).  Slots are reset in bulk by the
+// runtime before each drive (one cudaMemsetAsync), so no per-task reset is issued.
+#pragma once
+#include <stdint.h>
+
+#include "kernels.hpp"
+
+namespace vsk {
+
+__device__ __forceinline__ unsigned long long globaltimer_ns()
+{
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+    return t;
+}
+
+__device__ __forceinline__ void ctx_begin(const TaskCtx &c)
+{
+    // slot[0] keeps ~start so that max(~t) == min(t) and an all-zero slot is "empty"
+    if (c.slot && threadIdx.x == 0) atomicMax(&c.slot[0], ~globaltimer_ns());
+}
+
+// Call once per CTA, by all threads of the CTA, on every exit path (after the CTA's
+// last global store).
+__device__ __forceinline__ void ctx_end(const TaskCtx &c)
+{
+    if (!c.slot) return;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        atomicMax(&c.slot[1], globaltimer_ns());
+        const unsigned long long nct = (unsigned long long)gridDim.x * gridDim.y * gridDim.z;
+        if (atomicAdd(&c.slot[2], 1ull) == nct - 1) {
+            __threadfence();
+            const unsigned long long s = atomicAdd(&c.slot[0], 0ull), e = atomicAdd(&c.slot[1], 0ull);
+            if (c.host) {
+                volatile unsigned long long *h = c.host;
+                h[0] = s;
+                h[1] = e;
+            }
+            atomicExch(&c.slot[2], 0ull);   // re-arm for the task's next kernel
+        }
+    }
+}
+
+}  // namespace vsk

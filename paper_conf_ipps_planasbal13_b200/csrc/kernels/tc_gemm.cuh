@@ -28,6 +28,7 @@
 #include <stdint.h>
 
 #include "kernels.hpp"
+#include "task_ctx.cuh"
 
 namespace vsk {
 namespace tc {
@@ -164,8 +165,9 @@ __device__ __forceinline__ void store_split(uint8_t *big, uint8_t *small, uint32
 template <int BN, bool NT, bool NEG, bool LOWER>
 __global__ void __launch_bounds__(NTHREADS, 1)
 tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const float *__restrict__ B, int ldb,
-               float *__restrict__ C, int ldc)
+               float *__restrict__ C, int ldc, TaskCtx ctx)
 {
+    ctx_begin(ctx);
     using G = Cfg<BN>;
     constexpr int STAGES = G::STAGES;
     extern __shared__ uint8_t smem_raw[];
@@ -177,7 +179,10 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     uint32_t *tmem_slot = (uint32_t *)(c_ready + 1);
 
     const int m0 = blockIdx.y * BM, n0 = blockIdx.x * BN;
-    if (LOWER && n0 >= m0 + BM) return;
+    if (LOWER && n0 >= m0 + BM) {
+        ctx_end(ctx);
+        return;
+    }
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int nk = K / BK;
 
@@ -363,12 +368,13 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
         tc_fence_after();
         asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)BN));
     }
+    ctx_end(ctx);
 }
 
 // Host launcher: K multiple of 32; lda/ldb/ldc multiples of 4 and 16-byte aligned bases.
 template <bool NT, bool NEG, bool LOWER, int BN = 256>
 inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B, int ldb, float *C, int ldc,
-                   cudaStream_t s)
+                   cudaStream_t s, const TaskCtx &ctx = TaskCtx())
 {
     if (M <= 0 || N <= 0) return 0;
     if (K % BK) return -1;
@@ -383,7 +389,7 @@ inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B,
     }
     dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
     count_launch();
-    kern<<<grid, NTHREADS, smem, s>>>(M, N, K, A, lda, B, ldb, C, ldc);
+    kern<<<grid, NTHREADS, smem, s>>>(M, N, K, A, lda, B, ldb, C, ldc, ctx);
     return 0;
 }
 

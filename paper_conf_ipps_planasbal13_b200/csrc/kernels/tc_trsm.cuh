@@ -57,8 +57,9 @@ __device__ __forceinline__ float4 ld_f4_coherent(const float *p)
 }
 
 __global__ void __launch_bounds__(NTHREADS, 1)
-tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, int ldx)
+tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, int ldx, TaskCtx ctx)
 {
+    ctx_begin(ctx);
     using G = TrsmCfg;
     constexpr int P = TRSM_P, STAGES = G::STAGES;
     extern __shared__ uint8_t smem_raw[];
@@ -242,9 +243,11 @@ tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, 
     if (warp == NPROD / 32) {
         asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)P));
     }
+    ctx_end(ctx);
 }
 
-inline int tc_trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s)
+inline int tc_trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s,
+                   const TaskCtx &ctx = TaskCtx())
 {
     if (rows <= 0 || n <= 0) return 0;
     if (n % TRSM_P) return -1;
@@ -257,7 +260,7 @@ inline int tc_trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, 
         attr[dev & 63] = true;
     }
     count_launch();
-    tc_trsm_kernel<<<(rows + BM - 1) / BM, NTHREADS, smem, s>>>(rows, n, L, ldl, X, ldx);
+    tc_trsm_kernel<<<(rows + BM - 1) / BM, NTHREADS, smem, s>>>(rows, n, L, ldl, X, ldx, ctx);
     return 0;
 }
 

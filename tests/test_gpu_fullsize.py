@@ -57,7 +57,7 @@ def test_fullsize_bench_configuration(gpu):
     x = rng.standard_normal(Nc)
     Ax = A.astype(np.float64) @ x
     L64 = L.astype(np.float64)
-    assert np.linalg.norm(Ax - L64 @ (L64.T @ x)) / np.linalg.norm(Ax) <= 1e-5
+    assert np.linalg.norm(Ax - L64 @ (L64.T @ x)) / np.linalg.norm(Ax) <= 4 * Nc * 2.0 ** -24   # P3
     st = rt.vs_stats()
     assert st.tasks_completed == 2 * (4096 + 5984)
     rt.close()

@@ -119,10 +119,10 @@ def test_cfg2_cholesky_versioning(gpu):
     assert oracle.relF(L[:k, :k][slo], Lk[slo]) <= 1e-5
     rng = np.random.default_rng(0)
     A64, L64 = A.astype(np.float64), L.astype(np.float64)
-    for _ in range(4):
+    for _ in range(4):     # P3 reconstruction bound for fp32 factors: 4 N u, u = 2^-24
         x = rng.standard_normal(4096)
         r = A64 @ x - L64 @ (L64.T @ x)
-        assert np.linalg.norm(r) / np.linalg.norm(A64 @ x) <= 1e-5
+        assert np.linalg.norm(r) / np.linalg.norm(A64 @ x) <= 4 * 4096 * 2.0 ** -24
     gs = {g["type_name"]: g for g in rt.vs_group_stats()}
     assert not gs["POTRF.f32"]["reliable"] and sum(gs["POTRF.f32"]["n"]) == 8     # L496-501
     assert gs["GEMM_NT.f32"]["reliable"] and sum(gs["GEMM_NT.f32"]["n"]) == 56
