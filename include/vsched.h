@@ -113,12 +113,20 @@ typedef struct {
                           measurements (bit-exact decisions, P8).  Implied by VS_EXEC_SIM. */
     int flush;         /* 1 (default): vs_wait_all copies written data back to its home
                           (OmpSs flush, L264-270) */
+    int lookahead;     /* run-ahead window: at most this many issued-but-unfinished tasks
+                          per GPU (0 = unlimited).  Keeps worker queues short so a task on
+                          the critical path is not queued behind far-ahead work. */
+    int priority;      /* 0: ready tasks in submission order (R15, paper-literal);
+                          1: critical-path first (NEXT-4): ready order POTRF < TRSM < SYRK <
+                          GEMM_NT < MATMUL < user types, and POTRF/TRSM/SYRK launched on a
+                          high-priority stream of their worker (L711-718: potrf must run as
+                          soon as it is ready) */
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,
  * run-ahead, live timing, flush.  Environment overrides applied by vs_create (L277-288):
  * VS_LAMBDA, VS_SLOTS, VS_POLICY(=versioning|fixed:<v>), VS_LEARNING(=hold|rr),
- * VS_MODE(=runahead|ready). */
+ * VS_MODE(=runahead|ready), VS_LOOKAHEAD(=n), VS_PRIORITY(=0|1). */
 void vs_config_default(vs_config *cfg);
 
 /* Create a runtime.  *out receives an opaque handle owning scheduler state, DAG,

@@ -17,8 +17,11 @@
 //   warp 8     TMEM allocator + MMA issuer: one lane waits full[s], issues 3 x (BK/8)
 //              tcgen05.mma, tcgen05.commit -> empty[s]; after the last k-block,
 //              commit -> acc_full.
-//   warps 0-7  epilogue: warp w reads TMEM lanes 32(w%4).. (tile rows) and column half
-//              w/4 with tcgen05.ld 32x32b.x32, C += acc (fp32 RN), vector stores.
+//   warps 0-7  C_in prefetch: before the main loop each producer warp copies its part of
+//              the C tile (TMEM lanes 32(w%4).., column half w/4) into TMEM columns
+//              [BN, 2BN) with tcgen05.st, overlapping the first operand loads.
+//   warps 0-7  epilogue: tcgen05.ld of the accumulator and of C_in, C = C_in + acc in fp32
+//              round-to-nearest, vector stores (no global loads in the epilogue).
 // LOWER (syrk / potrf update): CTAs strictly above the diagonal exit; diagonal tiles
 // store only j <= i.
 // The MN-major B encoding (no transpose) was probed on B200 (tools/probe_mn.cu): with the
@@ -197,7 +200,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     }
     if (warp == NPROD / 32) {
         asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(tmem_slot)),
-                     "r"((uint32_t)BN));
+                     "r"((uint32_t)(2 * BN)));
         asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
     }
     tc_fence_before();
@@ -293,7 +296,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                 const float4 x = (erow < M && n0 + col0 + 4 * j < N) ? *reinterpret_cast<const float4 *>(crow + 4 * j) : z4;
                 v[4 * j] = x.x; v[4 * j + 1] = x.y; v[4 * j + 2] = x.z; v[4 * j + 3] = x.w;
             }
-            tmem_st32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)col0, v);
+            tmem_st32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(BN + col0), v);
         }
         asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
         tc_fence_before();
@@ -310,12 +313,17 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
         // ------------------------------------------------------------ epilogue
         mbar_wait(acc_full, 0);
         tc_fence_after();
-        // C was preloaded into the accumulator: store-only epilogue
+        // C_in was staged in TMEM columns [BN, 2BN): C = C_in + acc in fp32 round-to-nearest
+        // (the accumulation onto C is NOT done by the MMA: the tensor core's fp32
+        // accumulate is not round-to-nearest and loses precision on a large addend).
 #pragma unroll 1
         for (int c = 0; c < BN / 64; c++) {
             const int col0 = eh * (BN / 2) + c * 32;
-            float v[32];
+            float v[32], cv[32];
             tmem_ld32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)col0, v);
+            tmem_ld32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(BN + col0), cv);
+#pragma unroll
+            for (int i = 0; i < 32; i++) v[i] = cv[i] + v[i];
             if (erow < M) {
                 float *crow = C + (int64_t)erow * ldc + n0 + col0;
 #pragma unroll
@@ -338,7 +346,6 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
         constexpr uint32_t idesc = make_idesc(BM, BN, NEG, false);
         for (int kb = 0; kb < nk; kb++) {
             const int s = kb % STAGES;
-            if (kb == 0) mbar_wait(c_ready, 0);
             mbar_wait(&full[s], (kb / STAGES) & 1);
             tc_fence_after();
             if (lane == 0) {
@@ -351,7 +358,8 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                     const uint32_t o = kk * 32;
                     const uint64_t dAb = make_desc(a_big + o, 16, 1024), dAs = make_desc(a_small + o, 16, 1024);
                     const uint64_t dBb = make_desc(b_big + o, 16, 1024), dBs = make_desc(b_small + o, 16, 1024);
-                    mma_tf32(tmem, dAb, dBb, idesc, 1u);   // accumulate onto the preloaded C
+                    const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
+                    mma_tf32(tmem, dAb, dBb, idesc, first);
                     mma_tf32(tmem, dAb, dBs, idesc, 1u);
                     mma_tf32(tmem, dAs, dBb, idesc, 1u);
                 }
@@ -366,7 +374,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     __syncthreads();
     if (warp == NPROD / 32) {
         tc_fence_after();
-        asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)BN));
+        asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)(2 * BN)));
     }
     ctx_end(ctx);
 }
