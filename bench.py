@@ -426,6 +426,8 @@ def main():
                          "how": "hardware MMA flops (3x algorithmic) of all launches of this kernel class in the "
                                 "timed steps / union of their CUDA-event intervals on the worker streams"},
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
+            "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
+            "runtime_options": {"lookahead": rt.cfg.lookahead, "priority": rt.cfg.priority, "mode": rt.cfg.mode},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
             "host_us_per_task": {"decide": round((st1.host_ns_decide - st0.host_ns_decide) / 1e3 / max(1, len(log)), 3),

@@ -195,6 +195,8 @@ typedef struct {
     int64_t host_ns_issue;    /* host time spent issuing GPU work */
     int64_t virtual_now_ns;   /* DES clock */
     int64_t kernel_launches;  /* process-wide count of libvsched kernel launches */
+    int64_t tracker;          /* dependence tracker in use: 1 = device completion words
+                                 (stream memory operations), 0 = CUDA events */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 

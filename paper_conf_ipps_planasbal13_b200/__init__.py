@@ -46,7 +46,7 @@ class vs_stats_t(Structure):
     _fields_ = [(n, c_int64) for n in (
         "tasks_submitted", "tasks_completed", "decisions", "input_tx_bytes", "output_tx_bytes", "device_tx_bytes",
         "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns",
-        "kernel_launches")]
+        "kernel_launches", "tracker")]
 
 
 class vs_group_stat_t(Structure):
