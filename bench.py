@@ -287,7 +287,12 @@ def main():
 
     mm_n, mm_b, ch_n, ch_b = (MM_N, MM_B, CH_N, CH_B) if not args.small else (1024, 256, 4096, 512)
     with_mm, with_ch = args.only in ("mm", "both"), args.only in ("ch", "both")
-    cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0)
+    # critical-path priority (NEXT-4, vs_config.priority) is on by default in the bench;
+    # VS_PRIORITY=0 reproduces the paper-literal FIFO ready order (R15)
+    prio = int(os.environ.get("VS_PRIORITY", "1"))
+    look = int(os.environ.get("VS_LOOKAHEAD", "0"))
+    cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0,
+                               priority=prio, lookahead=look)
     rt = vs.Runtime(cfg)
     wl = Workload(rt, mm_n, mm_b, ch_n, ch_b, host=False, seed_off=rank, with_mm=with_mm, with_ch=with_ch)
     if args.table_load:
@@ -370,7 +375,7 @@ def main():
     # ---- e2e: same step through the C ABI with HOST (pinned) buffers, copies inside the timed region
     e2e = None
     if not args.no_e2e:
-        rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots))
+        rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look))
         wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, seed_off=rank, with_mm=with_mm, with_ch=with_ch)
         wl2.step()     # warm-up incl. learning
         tsum, h2d, d2h = 0.0, 0, 0
@@ -427,7 +432,8 @@ def main():
                                 "timed steps / union of their CUDA-event intervals on the worker streams"},
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
             "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
-            "runtime_options": {"lookahead": rt.cfg.lookahead, "priority": rt.cfg.priority, "mode": rt.cfg.mode},
+            "runtime_options": {"lookahead": look, "priority": prio, "mode": "runahead",
+                                "tracker_env": os.environ.get("VS_TRACKER", "memops")},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
             "host_us_per_task": {"decide": round((st1.host_ns_decide - st0.host_ns_decide) / 1e3 / max(1, len(log)), 3),
