@@ -9,11 +9,13 @@ completion by vs_wait_all: registration -> dependence analysis -> versioning dec
 
   python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
 
-value  = (2*16384^3 + 32768^3/3) flops per step x steps x ranks / max-over-ranks time.
-N > 1: one process per GPU (torchrun); each rank runs an independent instance of the
-step on its own GPU (weak scaling, no data-path collective).
---impl reference: the CPU oracle (oracle/) timed on this host's cores on a bounded
-sample of the same workload (the tier's reference arm).
+value = (2*16384^3 + 32768^3/3) algorithmic flops per step x steps / max-over-ranks time.
+N > 1 (torchrun, one process per GPU): the SAME problem is sharded (strong scaling):
+every tile has an owner rank (2D block-cyclic), every task runs on the owner of the tile
+it writes, and tiles owned by another rank are pulled over NVLink from the owner's memory
+(CUDA IPC) after the producer's completion tag is visible (vs_dist_init).
+--impl reference: the CPU oracle (oracle/) timed on this host's cores on a bounded sample
+of the same workload (this tier's reference arm).
 """
 from __future__ import annotations
 
@@ -45,67 +47,98 @@ def peaks():
     return {"hbm_gbs": 6650.0, "bf16_tflops": 1590.0, "bf16_tflops_sustained": 1400.0, "sm_max_mhz": 1965.0}, "fallback"
 
 
+def rank_grid(nranks):
+    """P_r x P_c process grid for the 2D block-cyclic tile ownership (§8(e))."""
+    return {1: (1, 1), 2: (1, 2), 4: (2, 2), 8: (2, 4)}.get(nranks, (1, nranks))
+
+
+def tile_owner(i, j, nranks):
+    pr, pc = rank_grid(nranks)
+    return (i % pr) * pc + (j % pc)
+
+
 # ----------------------------------------------------------------------------- workload
 class Workload:
-    """Device-resident (or pinned-host, for e2e) tiles of cfg3 + cfg4 and their data ids."""
+    """Tiles of cfg3 + cfg4 and their data ids.  Each rank allocates and generates only the
+    tiles it owns (vs_gen_tile, bit-identical to vsgen); with nranks > 1 the other ranks'
+    tiles are opened through CUDA IPC and registered as owned by them.  host=True (e2e,
+    one rank) keeps the tiles in pinned host memory and lets the runtime move them."""
 
-    def __init__(self, rt, mm_n=MM_N, mm_b=MM_B, ch_n=CH_N, ch_b=CH_B, host=False, seed_off=0, mask=F32_VERSIONS_MASK,
-                 with_mm=True, with_ch=True):
+    def __init__(self, rt, mm_n=MM_N, mm_b=MM_B, ch_n=CH_N, ch_b=CH_B, host=False, rank=0, nranks=1, gather=None,
+                 mask=F32_VERSIONS_MASK, with_mm=True, with_ch=True):
         import torch
         import paper_conf_ipps_planasbal13_b200 as vs
         self.torch, self.vs, self.rt = torch, vs, rt
         self.mm_n, self.mm_b, self.ch_n, self.ch_b, self.host = mm_n, mm_b, ch_n, ch_b, host
+        self.rank, self.nranks = rank, nranks
         self.with_mm, self.with_ch = with_mm, with_ch
         self.types = rt.vs_register_builtins(vs.VS_F32, mask)
-        dev = torch.device("cuda")
-        dev_i = -1 if host else 0
         self.flops = 0.0
+        self.ids = []            # every registered datum (for invalidation)
+        self.opened = []         # IPC bases to close
         if with_mm:
             nt = mm_n // mm_b
             self.mm_nt = nt
-            # generated on the device by vs_gen_uniform (bit-identical to vsgen)
-            gA = torch.empty((nt, nt, mm_b, mm_b), dtype=torch.float32, device=dev)
-            gB = torch.empty_like(gA)
-            vs.vs_gen_uniform(SEED_MM + seed_off, mm_n, mm_n, vs.VS_F32, mm_b, gA.data_ptr())
-            vs.vs_gen_uniform(SEED_MM + 1000 + seed_off, mm_n, mm_n, vs.VS_F32, mm_b, gB.data_ptr())
-            if host:
-                self.A = gA.cpu().pin_memory()
-                self.B = gB.cpu().pin_memory()
-                self.C = torch.zeros_like(self.A).pin_memory()
-                del gA, gB
-            else:
-                self.A, self.B = gA, gB
-                self.C = torch.zeros_like(gA)
-            nb = mm_b * mm_b * 4
-            reg = lambda T: [rt.vs_data_register(T[i, j].data_ptr(), dev_i, nb) for i in range(nt) for j in range(nt)]  # noqa
-            self.ia, self.ib, self.ic = reg(self.A), reg(self.B), reg(self.C)
+            all_t = [(i, j) for i in range(nt) for j in range(nt)]
+            self.A, self.ia = self._matrix("A", all_t, mm_b, mm_n, lambda T, k, i, j: vs.vs_gen_tile(
+                SEED_MM, mm_n, mm_n, vs.VS_F32, mm_b, i, j, 0, T[k].data_ptr()), gather)
+            self.B, self.ib = self._matrix("B", all_t, mm_b, mm_n, lambda T, k, i, j: vs.vs_gen_tile(
+                SEED_MM + 1000, mm_n, mm_n, vs.VS_F32, mm_b, i, j, 0, T[k].data_ptr()), gather)
+            self.C, self.ic = self._matrix("C", all_t, mm_b, mm_n, None, gather)
             self.flops += MM_FLOPS(mm_n)
         if with_ch:
             nt = ch_n // ch_b
             self.ch_nt = nt
-            g = torch.empty((nt, nt, ch_b, ch_b), dtype=torch.float32, device=dev)
-            vs.vs_gen_spd(SEED_CH + seed_off, ch_n, vs.VS_F32, ch_b, g.data_ptr())
-            if host:
-                self.S0 = g.cpu()
-                self.S = self.S0.clone().pin_memory()
-                del g
-            else:
-                self.S0 = g
-                self.S = g.clone()
-            nb = ch_b * ch_b * 4
-            self.iS = {i * nt + j: rt.vs_data_register(self.S[i, j].data_ptr(), dev_i, nb)
-                       for i in range(nt) for j in range(i + 1)}
+            low = [(i, j) for i in range(nt) for j in range(i + 1)]
+            self.S, idl = self._matrix("S", low, ch_b, ch_n, lambda T, k, i, j: vs.vs_gen_tile(
+                SEED_CH, ch_n, ch_n, vs.VS_F32, ch_b, i, j, 1, T[k].data_ptr()), gather)
+            self.S0 = self.S.clone()
+            self.iS = {i * nt + j: d for (i, j), d in zip(low, idl)}
             self.flops += CH_FLOPS(ch_n)
         torch.cuda.synchronize()
 
+    def _matrix(self, name, tiles, b, n, gen, gather):
+        """Allocate this rank's tiles of one matrix (one buffer), register every tile."""
+        torch, vs, rt = self.torch, self.vs, self.rt
+        own = [t for t in tiles if tile_owner(t[0], t[1], self.nranks) == self.rank]
+        T = torch.zeros((max(1, len(own)), b, b), dtype=torch.float32, device="cuda")
+        if gen is not None:
+            for k, (i, j) in enumerate(own):
+                gen(T, k, i, j)
+        if self.host:
+            T = T.cpu().pin_memory()
+        nbytes = b * b * 4
+        dev = -1 if self.host else 0
+        ids = {}
+        for k, t in enumerate(own):
+            ids[t] = rt.vs_data_register(T[k].data_ptr(), dev, nbytes)
+        if self.nranks > 1:
+            h, off = vs.vs_ipc_export(T.data_ptr())
+            peers = gather((self.rank, h, off, own))
+            for (r, hr, offr, ownr) in peers:
+                if r == self.rank:
+                    continue
+                base = vs.vs_ipc_open(hr, offr)
+                self.opened.append(base - offr)
+                for k, t in enumerate(ownr):
+                    d = rt.vs_data_register(base + k * nbytes, 0, nbytes)
+                    rt.vs_data_set_owner(d, r)
+                    ids[t] = d
+        self.ids.extend(ids.values())
+        return T, [ids[t] for t in tiles]
+
     def reset(self):
-        """Restore the step's inputs (C = 0, A_chol = pristine).  Device: async on torch's
-        stream + sync; host: memcpy (outside the timed region for e2e)."""
+        """Restore this rank's inputs (C = 0, A_chol = pristine).  Device: async on torch's
+        stream + sync.  Host (e2e): memcpy, then every datum is declared modified so the
+        runtime re-transfers it (the e2e timed region includes those copies)."""
         if self.with_mm:
             self.C.zero_()
         if self.with_ch:
             self.S.copy_(self.S0)
-        if not self.host:
+        if self.host:
+            for d in self.ids:
+                self.rt.vs_data_invalidate(d)
+        else:
             self.torch.cuda.current_stream().synchronize()
 
     def submit(self):
@@ -116,8 +149,10 @@ class Workload:
         if self.with_ch:
             rt.vs_app_cholesky(self.types, self.ch_nt, self.iS)
 
-    def step(self):
+    def step(self, barrier=None):
         self.reset()
+        if barrier:
+            barrier()      # owners' resets done before any rank reads their tiles
         self.submit()
         self.rt.vs_wait_all()
 
@@ -185,7 +220,45 @@ def task_flops(type_name, b):
             "POTRF": b ** 3 / 3.0}[t]
 
 
+def roofline(log, groups, ms, world):
+    pk, pk_kind = peaks()
+    tf32_peak = pk.get("bf16_tflops_sustained", pk["bf16_tflops"]) * 0.5   # TF32 = 1/2 BF16 (nominal ratio)
+    tnames = {g["type"]: g["type_name"] for g in groups}
+    vnames = {g["type"]: g["versions"] for g in groups}
+    tile_b = {}
+    for g in groups:
+        npar = {"MATMUL": 3, "GEMM_NT": 3, "SYRK": 2, "TRSM": 2, "POTRF": 1}[g["type_name"].split(".")[0]]
+        tile_b[g["type"]] = int(round(math.sqrt(g["bytes"] / 4 / npar)))
+    per = {}
+    for (task, v, w, td, ts, te, ph, ty) in log:
+        key = (tnames[ty], vnames[ty][v], tile_b[ty])
+        d = per.setdefault(key, {"n": 0, "flops": 0.0, "iv": []})
+        d["n"] += 1
+        d["flops"] += task_flops(tnames[ty], tile_b[ty])
+        d["iv"].append((ts, te))
+    dom = max(per, key=lambda k: per[k]["flops"])
+    d = per[dom]
+    union = union_ns(d["iv"])
+    hw = 3.0 if dom[1] == "tc_3xtf32" else 1.0
+    achieved = hw * d["flops"] / (union * 1e-9) / 1e12
+    if dom[1] == "tc_3xtf32":
+        peak, bound, src = tf32_peak, "tensor", "%s bf16_tflops_sustained x 0.5 (TF32/BF16 nominal ratio)" % pk_kind
+    else:
+        peak, bound, src = 148 * 128 * 2 * pk["sm_max_mhz"] * 1e6 / 1e12, "alu", "148 SM x 128 FMA x 2 x sm_max_mhz"
+    tc_flops = sum(v["flops"] for k, v in per.items() if k[1] == "tc_3xtf32")
+    frac_step = 3.0 * tc_flops / (ms * 1e-3) / 1e12 / tf32_peak
+    roof = {"bound": bound, "kernel": "%s/%s b=%d" % dom, "achieved": round(achieved, 2), "peak": round(peak, 1),
+            "unit": "TFLOP/s", "frac": round(achieved / peak, 4), "traffic": None, "peak_source": src,
+            "how": "hardware MMA flops (3x algorithmic) of all launches of this kernel class in the timed steps / "
+                   "union of their device-recorded execution intervals (%globaltimer, task_ctx.cuh)"}
+    counts = {"%s/%s" % k[:2]: v["n"] for k, v in sorted(per.items())}
+    return roof, frac_step, counts
+
+
 # ----------------------------------------------------------------------------- reference arm
+_CPU = {}
+
+
 def cpu_sample(target_s=12.0):
     """The oracle as it stands, on a bounded sample of the same workload:
     matmul rows 0..R-1 of C = A*B at N=16384 (fp64, plain i,k,j loop) and the Cholesky of
@@ -196,31 +269,28 @@ def cpu_sample(target_s=12.0):
     import vsgen
     cores = len(os.sched_getaffinity(0))
     os.environ.setdefault("OMP_NUM_THREADS", str(cores))
-    # calibrate rows: one row of C costs 2*N^2 flops
-    A_rows = vsgen.uniform(SEED_MM, 64, MM_N)
-    B = vsgen.uniform_idx(SEED_MM + 1000, np.arange(MM_N * MM_N, dtype=np.uint64)).reshape(MM_N, MM_N)
+    if "B" not in _CPU:    # input generation is not part of the timed oracle work
+        _CPU["A"] = vsgen.uniform(SEED_MM, 64, MM_N).astype(np.float64)
+        _CPU["B"] = vsgen.uniform_idx(SEED_MM + 1000, np.arange(MM_N * MM_N, dtype=np.uint64)).reshape(MM_N, MM_N)
+        k = 2048
+        r = np.arange(k, dtype=np.uint64)[:, None]
+        c = np.arange(k, dtype=np.uint64)[None, :]
+        S = vsgen.uniform_idx(SEED_CH, np.maximum(r, c) * np.uint64(CH_N) + np.minimum(r, c))
+        S[np.arange(k), np.arange(k)] += vsgen.spd_alpha(CH_N)
+        _CPU["S"] = S.astype(np.float32).astype(np.float64)
+        t0 = time.perf_counter()
+        oracle.matmul(_CPU["A"][:4], _CPU["B"])
+        _CPU["dt_row"] = (time.perf_counter() - t0) / 4
+    rows = int(max(4, min(64, (target_s / 2) / max(_CPU["dt_row"], 1e-4))))
     t0 = time.perf_counter()
-    oracle.matmul(A_rows[:8], B)
-    dt8 = time.perf_counter() - t0
-    rows = int(max(8, min(64, 8 * (target_s / 2) / max(dt8, 1e-3))))
-    t0 = time.perf_counter()
-    oracle.matmul(A_rows[:rows], B)
+    oracle.matmul(_CPU["A"][:rows], _CPU["B"])
     t_mm = time.perf_counter() - t0
-    f_mm = 2.0 * rows * MM_N * MM_N
-    k = 2048
-    # leading k x k block of the N=32768 SPD matrix (same generator, global indices)
-    r = np.arange(k, dtype=np.uint64)[:, None]
-    c = np.arange(k, dtype=np.uint64)[None, :]
-    hi, lo = np.maximum(r, c), np.minimum(r, c)
-    S = vsgen.uniform_idx(SEED_CH, hi * np.uint64(CH_N) + lo)
-    S[np.arange(k), np.arange(k)] += vsgen.spd_alpha(CH_N)
-    S = S.astype(np.float32)
+    k = _CPU["S"].shape[0]
     t0 = time.perf_counter()
-    _, info = oracle.cholesky(S)
+    _, info = oracle.cholesky(_CPU["S"])
     t_ch = time.perf_counter() - t0
-    f_ch = k ** 3 / 3.0
-    return {"t_mm": t_mm, "f_mm": f_mm, "rows": rows, "t_ch": t_ch, "f_ch": f_ch, "k": k, "cores": cores,
-            "info": info}
+    return {"t_mm": t_mm, "f_mm": 2.0 * rows * MM_N * MM_N, "rows": rows, "t_ch": t_ch, "f_ch": k ** 3 / 3.0,
+            "k": k, "cores": cores, "info": info}
 
 
 def run_reference(args, rank, world):
@@ -239,8 +309,9 @@ def run_reference(args, rank, world):
               "leading %dx%d block of the cfg4 SPD matrix" % (s0["rows"] - 1, s0["k"], s0["k"]))
     out = {"metric": "tiled matmul & Cholesky GFLOP/s", "value": round(gf, 3), "unit": "GFLOP/s", "impl": "reference",
            "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
-           "ms_per_step": round(1e3 * t / len(samples), 2), "higher_is_better": True, "scaling": "weak",
-           "vs_baseline": None, "dtype": "f64", "data": "synthetic (vsgen counter-based generator)",
+           "ms_per_step": round(1e3 * t / len(samples), 2), "higher_is_better": True,
+           "scaling": "strong" if world > 1 else "weak", "vs_baseline": None, "dtype": "f64",
+           "data": "synthetic (vsgen counter-based generator)",
            "config": {"workload": "cfg3+cfg4 (bounded CPU sample)", "matmul_N": MM_N, "cholesky_N": CH_N},
            "cpu_baseline": {"value": round(gf, 3), "unit": "GFLOP/s", "cores": s0["cores"], "kind": "oracle",
                             "sample": sample},
@@ -275,15 +346,21 @@ def main():
 
     import torch
     import paper_conf_ipps_planasbal13_b200 as vs
-    torch.cuda.set_device(local)
+    ndev = torch.cuda.device_count()
+    torch.cuda.set_device(local % max(1, ndev))
     dist = None
     if world > 1:
         import torch.distributed as dist
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        dist.init_process_group("gloo")   # host-side plumbing only (IPC handles, barriers, max)
 
     def barrier():
         if dist is not None:
             dist.barrier()
+
+    def gather(obj):
+        out = [None] * world
+        dist.all_gather_object(out, obj)
+        return out
 
     mm_n, mm_b, ch_n, ch_b = (MM_N, MM_B, CH_N, CH_B) if not args.small else (1024, 256, 4096, 512)
     with_mm, with_ch = args.only in ("mm", "both"), args.only in ("ch", "both")
@@ -294,7 +371,16 @@ def main():
     cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0,
                                priority=prio, lookahead=look)
     rt = vs.Runtime(cfg)
-    wl = Workload(rt, mm_n, mm_b, ch_n, ch_b, host=False, seed_off=rank, with_mm=with_mm, with_ch=with_ch)
+    if world > 1:
+        shm = gather("/vsched_%d_%d" % (os.getpid(), int(time.time())) if rank == 0 else None)[0]
+        if rank == 0:
+            rt.vs_dist_init(rank, world, shm)
+        barrier()
+        if rank != 0:
+            rt.vs_dist_init(rank, world, shm)
+        barrier()
+    wl = Workload(rt, mm_n, mm_b, ch_n, ch_b, host=False, rank=rank, nranks=world, gather=gather if world > 1 else None,
+                  with_mm=with_mm, with_ch=with_ch)
     if args.table_load:
         rt.vs_table_load(args.table_load)
         if args.replay:          # replay durations = the loaded means
@@ -305,19 +391,23 @@ def main():
                         vi = [vs.lib().vs_version_name(rt.h, ti, v).decode() for v in range(8)
                               if vs.lib().vs_version_name(rt.h, ti, v)].index(vn)
                         rt.vs_replay_set(ti, int(nb), vi, int(mean))
+    step_barrier = barrier if world > 1 else None
 
     # warm-up (the first step includes the learning phase: "cold")
+    barrier()
     t0 = time.perf_counter()
-    wl.step()
+    wl.step(step_barrier)
+    barrier()
     cold_ms = (time.perf_counter() - t0) * 1e3
     for _ in range(args.warmup - 1):
-        wl.step()
+        wl.step(step_barrier)
     if args.table_dump:
         rt.vs_table_dump(args.table_dump)
+    barrier()
     rt.vs_decision_log_clear()
     st0 = rt.vs_stats()
 
-    sampler = ClockSampler(local)
+    sampler = ClockSampler(torch.cuda.current_device())
     sampler.start()
     time.sleep(0.3)
     barrier()
@@ -325,68 +415,39 @@ def main():
     ev0, ev1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     ev0.record()
     for _ in range(args.steps):
-        wl.step()
+        wl.step(step_barrier)
+    barrier()
     ev1.record()
     torch.cuda.synchronize()
-    barrier()
     ms = ev0.elapsed_time(ev1)
     clocks = sampler.stop()
     if dist is not None:
-        t = torch.tensor([ms], device="cuda")
-        dist.all_reduce(t, op=dist.ReduceOp.MAX)
-        ms = float(t.item())
+        ms = max(gather(ms))
     st1 = rt.vs_stats()
     log = rt.vs_decision_log()
     groups = rt.vs_group_stats()
     ms_step = ms / args.steps
-    gflops = wl.flops * args.steps * world / (ms * 1e-3) / 1e9
-
-    # ---- roofline of the dominant kernel (the (type, version) carrying most flops in the timed steps)
-    pk, pk_kind = peaks()
-    tf32_peak = pk.get("bf16_tflops_sustained", pk["bf16_tflops"]) * 0.5   # TF32 = 1/2 BF16 (nominal ratio)
-    tnames = {g["type"]: g["type_name"] for g in groups}
-    vnames = {g["type"]: g["versions"] for g in groups}
-    tile_b = {}
-    for g in groups:
-        npar = {"MATMUL": 3, "GEMM_NT": 3, "SYRK": 2, "TRSM": 2, "POTRF": 1}[g["type_name"].split(".")[0]]
-        tile_b[g["type"]] = int(round(math.sqrt(g["bytes"] / 4 / npar)))
-    per = {}
-    for (task, v, w, td, ts, te, ph, ty) in log:
-        key = (tnames[ty], vnames[ty][v])
-        d = per.setdefault(key, {"n": 0, "flops": 0.0, "iv": [], "busy_ns": 0})
-        d["n"] += 1
-        d["flops"] += task_flops(tnames[ty], tile_b[ty])
-        d["iv"].append((ts, te))
-        d["busy_ns"] += te - ts
-    dom = max(per, key=lambda k: per[k]["flops"])
-    d = per[dom]
-    union = union_ns(d["iv"])
-    hw = 3.0 if dom[1] == "tc_3xtf32" else 1.0
-    achieved = hw * d["flops"] / (union * 1e-9) / 1e12          # TFLOP/s while that kernel class runs
-    if dom[1] == "tc_3xtf32":
-        peak, unit, bound = tf32_peak, "TFLOP/s", "tensor"
-    else:
-        peak, unit, bound = 148 * 128 * 2 * pk["sm_max_mhz"] * 1e6 / 1e12, "TFLOP/s", "alu"
-    tc_flops = sum(v["flops"] for k, v in per.items() if k[1] == "tc_3xtf32")
-    tensor_frac_step = 3.0 * tc_flops / (ms * 1e-3 / world) / 1e12 / tf32_peak if world == 1 else None
-    version_counts = {"%s/%s" % k: v["n"] for k, v in sorted(per.items())}
+    gflops = wl.flops * args.steps / (ms * 1e-3) / 1e9       # one problem, sharded over the ranks
+    roof, frac_step, version_counts = roofline(log, groups, ms, 1)
     launches = st1.kernel_launches - st0.kernel_launches
+    if dist is not None:
+        launches = sum(gather(int(launches)))
 
     # ---- e2e: same step through the C ABI with HOST (pinned) buffers, copies inside the timed region
     e2e = None
-    if not args.no_e2e:
+    if not args.no_e2e and world == 1:
         rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look))
-        wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, seed_off=rank, with_mm=with_mm, with_ch=with_ch)
+        wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, with_mm=with_mm, with_ch=with_ch)
         wl2.step()     # warm-up incl. learning
         tsum, h2d, d2h = 0.0, 0, 0
         n_e2e = 2
         for _ in range(n_e2e):
-            wl2.reset()
+            wl2.reset()                      # host restore + invalidate (outside the timing)
             s0 = rt2.vs_stats()
             torch.cuda.synchronize()
             t0 = time.perf_counter()
             wl2.submit()
-            rt2.vs_wait_all()            # includes the flush of written tiles to host (Output Tx)
+            rt2.vs_wait_all()                # includes the flush of written tiles to host (Output Tx)
             torch.cuda.synchronize()
             tsum += time.perf_counter() - t0
             s1 = rt2.vs_stats()
@@ -410,7 +471,7 @@ def main():
         out = {
             "metric": "tiled matmul & Cholesky GFLOP/s", "value": round(gflops, 1), "unit": "GFLOP/s",
             "n_gpus": world, "steps": args.steps, "warmup": args.warmup, "ms_per_step": round(ms_step, 3),
-            "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f32",
+            "higher_is_better": True, "scaling": "strong" if world > 1 else "weak", "vs_baseline": None, "dtype": "f32",
             "data": "synthetic (counter-based generator; U(-1,1) matmul operands, SPD A = S + 2.5 sqrt(N) I)",
             "config": {"workload": ("cfg3+cfg4: tiled matmul N=%d b=%d + tiled Cholesky N=%d b=%d, fp32, versions "
                                     "simt_f32/tc_3xtf32/f64in_f32io, lambda=%d, %d slots/GPU" % (
@@ -418,30 +479,27 @@ def main():
                        args.only,
                        "matmul_N": mm_n if with_mm else None, "cholesky_N": ch_n if with_ch else None,
                        "tile": mm_b, "lambda": args.lam, "slots_per_gpu": args.slots,
-                       "parallelism": "independent instance per GPU" if world > 1 else "1 GPU",
-                       "l2": "inputs larger than L2 (4 GiB + 4 GiB per GPU)", "regime": "warm (tables learned in warm-up)"},
-            "parts_gflop": {"matmul": MM_FLOPS(mm_n) / 1e9 if with_mm else 0, "cholesky": CH_FLOPS(ch_n) / 1e9 if with_ch else 0},
+                       "parallelism": ("owner-computes 2D block-cyclic %dx%d, NVLink tile pulls" % rank_grid(world))
+                       if world > 1 else "1 GPU",
+                       "l2": "inputs larger than L2 (4 GiB + 4 GiB)", "regime": "warm (tables learned in warm-up)"},
+            "parts_gflop": {"matmul": MM_FLOPS(mm_n) / 1e9 if with_mm else 0,
+                            "cholesky": CH_FLOPS(ch_n) / 1e9 if with_ch else 0},
             "cold_first_step_ms": round(cold_ms, 1),
-            "tensor_pipe_fraction_step": round(tensor_frac_step, 4) if tensor_frac_step is not None else None,
-            "roofline": {"bound": bound, "kernel": "%s/%s b=%d" % (dom[0], dom[1], tile_b[[t for t in tnames if tnames[t] == dom[0]][0]]),
-                         "achieved": round(achieved, 2), "peak": round(peak, 1), "unit": unit,
-                         "frac": round(achieved / peak, 4), "traffic": None,
-                         "peak_source": "%s bf16_tflops_sustained x 0.5 (TF32/BF16 nominal ratio)" % pk_kind
-                         if bound == "tensor" else "148 SM x 128 FMA x 2 x sm_max_mhz",
-                         "how": "hardware MMA flops (3x algorithmic) of all launches of this kernel class in the "
-                                "timed steps / union of their CUDA-event intervals on the worker streams"},
+            "tensor_pipe_fraction_step": round(frac_step, 4) if world == 1 else None,
+            "roofline": roof,
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
             "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
-            "runtime_options": {"lookahead": look, "priority": prio, "mode": "runahead",
-                                "tracker_env": os.environ.get("VS_TRACKER", "memops")},
+            "runtime_options": {"lookahead": look, "priority": prio, "mode": "runahead"},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
+            "device_tx_bytes_per_step": int((st1.device_tx_bytes - st0.device_tx_bytes) / args.steps),
             "host_us_per_task": {"decide": round((st1.host_ns_decide - st0.host_ns_decide) / 1e3 / max(1, len(log)), 3),
                                  "issue": round((st1.host_ns_issue - st0.host_ns_issue) / 1e3 / max(1, len(log)), 3)},
         }
         print(json.dumps(out))
         if args.dump_log:
             json.dump({"log": log, "groups": groups}, open(args.dump_log, "w"))
+    barrier()
     rt.close()
     if dist is not None:
         dist.destroy_process_group()

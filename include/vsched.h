@@ -170,6 +170,11 @@ int vs_register_builtins(vs_rt rt, int dtype, uint32_t version_mask,
  * same id; a partial overlap with a registered region is VS_E_OVERLAP (R21). */
 int vs_data_register(vs_rt rt, void *ptr, int device, int64_t bytes, vs_data_id *out);
 
+/* The caller modified datum d at its home outside any task (after a wait): every other
+ * copy (device replica, cached remote copy) is stale and will be re-fetched on next use.
+ * VS_E_STATE if a task writing d is still in flight. */
+int vs_data_invalidate(vs_rt rt, vs_data_id d);
+
 /* ------------------------------------------------------------- submission (a2) */
 /* Create a task instance: RAW/WAR/WAW edges on whole data (L236-242).  scalars
  * (may be NULL) are copied and passed to the version.  Execution happens inside
@@ -274,6 +279,33 @@ int vs_gen_uniform(uint64_t seed, int64_t rows, int64_t cols, int dtype, int til
 /* SPD recipe R8: S_rc = u(seed, max(r,c)*n + min(r,c)); diagonal fl(S_rr + alpha) with
  * alpha = 2.5*sqrt(n) (n >= 256) else n, computed in fp64.  Layout as vs_gen_uniform. */
 int vs_gen_spd(uint64_t seed, int64_t n, int dtype, int tile_b, void *dev_out, void *stream);
+
+/* One tile_b x tile_b tile at global tile coordinates (ti, tj) of the rows x cols uniform
+ * matrix (spd = 0) or of the cols x cols SPD matrix (spd = 1), row-major, same values as
+ * vs_gen_uniform / vs_gen_spd (used by ranks that own only some tiles). */
+int vs_gen_tile(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b, int64_t ti, int64_t tj, int spd,
+                void *dev_out, void *stream);
+
+/* ------------------------------------------- one process per GPU */
+/* Join a job of nranks processes on one node as `rank`.  Every rank submits the SAME task
+ * graph; a task is executed only by the rank owning its written datum (owner computes,
+ * vs_data_set_owner), and is retired at once elsewhere.  A rank reading a datum owned by
+ * another rank copies it over NVLink from the owner's memory (a CUDA IPC pointer given at
+ * registration) after the producing task's completion tag is visible: tags live in the
+ * POSIX shared-memory segment shm_name (created by rank 0, which must call first; the
+ * binding orders the calls with a barrier) registered with every rank's GPU, so the wait
+ * is a stream memory operation on the device, with no host round trip.  Restrictions: run-
+ * ahead mode; a rank never overwrites a datum another rank may still be copying (true of
+ * vs_app_matmul / vs_app_cholesky with owner computes).  Must precede submissions. */
+int vs_dist_init(vs_rt rt, int rank, int nranks, const char *shm_name);
+/* Datum d is owned by rank `owner` (its pointer is then the owner's memory, opened with
+ * vs_ipc_open); data registered without this call belong to the calling rank. */
+int vs_data_set_owner(vs_rt rt, vs_data_id d, int owner);
+/* CUDA IPC without CUDA types: export a device pointer as a 64-byte handle + byte offset in
+ * its allocation; open a peer handle (pointer valid in this process); close an opened base. */
+int vs_ipc_export(const void *dev_ptr, unsigned char handle[64], uint64_t *offset);
+int vs_ipc_open(const unsigned char handle[64], uint64_t offset, void **dev_ptr);
+int vs_ipc_close(void *base_ptr);
 
 /* Library build information (never NULL). */
 const char *vs_build_info(void);

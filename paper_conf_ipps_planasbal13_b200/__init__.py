@@ -113,6 +113,13 @@ def lib():
         "vs_gen_uniform": (c_int, [c_uint64, c_int64, c_int64, c_int, c_int, c_void_p, c_void_p]),
         "vs_gen_spd": (c_int, [c_uint64, c_int64, c_int, c_int, c_void_p, c_void_p]),
         "vs_build_info": (c_char_p, []),
+        "vs_gen_tile": (c_int, [c_uint64, c_int64, c_int64, c_int, c_int, c_int64, c_int64, c_int, c_void_p, c_void_p]),
+        "vs_dist_init": (c_int, [rt, c_int, c_int, c_char_p]),
+        "vs_data_set_owner": (c_int, [rt, c_int64, c_int]),
+        "vs_ipc_export": (c_int, [c_void_p, ctypes.c_char * 64, POINTER(c_uint64)]),
+        "vs_ipc_open": (c_int, [ctypes.c_char * 64, c_uint64, POINTER(c_void_p)]),
+        "vs_ipc_close": (c_int, [c_void_p]),
+        "vs_data_invalidate": (c_int, [rt, c_int64]),
     }
     for name, (res, args) in sig.items():
         f = getattr(L, name)
@@ -127,7 +134,8 @@ EXPORTED = ["vs_config_default", "vs_create", "vs_destroy", "vs_last_error", "vs
             "vs_wait_on", "vs_stats", "vs_group_count", "vs_group_stat", "vs_type_name", "vs_version_name",
             "vs_decision_log", "vs_decision_log_hash", "vs_decision_log_clear", "vs_table_dump", "vs_table_load",
             "vs_replay_set", "vs_app_matmul", "vs_app_cholesky", "vs_tile_run", "vs_gen_uniform", "vs_gen_spd",
-            "vs_build_info"]
+            "vs_build_info", "vs_gen_tile", "vs_dist_init", "vs_data_set_owner", "vs_ipc_export", "vs_ipc_open",
+            "vs_ipc_close", "vs_data_invalidate"]
 
 
 def _ids(seq, ctype=c_int64):
@@ -166,6 +174,35 @@ def vs_gen_spd(seed, n, dtype, tile_b, dev_ptr, stream=0):
 
 def vs_build_info() -> str:
     return lib().vs_build_info().decode()
+
+
+def vs_gen_tile(seed, rows, cols, dtype, tile_b, ti, tj, spd, dev_ptr, stream=0):
+    r = lib().vs_gen_tile(seed, rows, cols, dtype, tile_b, ti, tj, spd, c_void_p(dev_ptr), c_void_p(stream or None))
+    if r:
+        raise VSError(r, "vs_gen_tile")
+
+
+def vs_ipc_export(dev_ptr):
+    """-> (64-byte handle as bytes, offset) of a device pointer."""
+    h = (ctypes.c_char * 64)()
+    off = c_uint64()
+    r = lib().vs_ipc_export(c_void_p(dev_ptr), h, ctypes.byref(off))
+    if r:
+        raise VSError(r, "vs_ipc_export")
+    return bytes(h.raw), off.value
+
+
+def vs_ipc_open(handle: bytes, offset: int) -> int:
+    h = (ctypes.c_char * 64).from_buffer_copy(handle)
+    p = c_void_p()
+    r = lib().vs_ipc_open(h, offset, ctypes.byref(p))
+    if r:
+        raise VSError(r, "vs_ipc_open")
+    return p.value
+
+
+def vs_ipc_close(base_ptr: int):
+    lib().vs_ipc_close(c_void_p(base_ptr))
 
 
 class Runtime:
@@ -284,6 +321,15 @@ class Runtime:
 
     def vs_replay_set(self, ttype, nbytes, version, ns):
         return self._ck(lib().vs_replay_set(self.h, ttype, nbytes, version, ns), "vs_replay_set")
+
+    def vs_data_invalidate(self, d):
+        return self._ck(lib().vs_data_invalidate(self.h, d), "vs_data_invalidate")
+
+    def vs_dist_init(self, rank, nranks, shm_name=""):
+        return self._ck(lib().vs_dist_init(self.h, rank, nranks, shm_name.encode()), "vs_dist_init")
+
+    def vs_data_set_owner(self, d, owner):
+        return self._ck(lib().vs_data_set_owner(self.h, d, owner), "vs_data_set_owner")
 
     def vs_app_matmul(self, mm_type, m, l, n, A, B, C):
         return self._ck(lib().vs_app_matmul(self.h, mm_type, m, l, n, _ids(A), _ids(B), _ids(C)), "vs_app_matmul")

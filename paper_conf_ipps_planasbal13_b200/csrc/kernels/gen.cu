@@ -83,3 +83,41 @@ int gen_spd(uint64_t seed, int64_t n, int dtype, int tile_b, void *out, cudaStre
 }
 
 }  // namespace vsk
+
+namespace vsk {
+
+// One b x b tile (global tile coordinates ti, tj) of a rows x cols uniform matrix, or of
+// the n x n SPD matrix (spd != 0): same values as the whole-matrix generators.
+template <typename T>
+__global__ void gen_tile_kernel(uint64_t seed, int64_t cols, int b, int64_t ti, int64_t tj, int spd, double alpha,
+                                T *out)
+{
+    const int64_t total = (int64_t)b * b;
+    for (int64_t e = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; e < total; e += (int64_t)gridDim.x * blockDim.x) {
+        const int64_t r = ti * b + e / b, c = tj * b + e % b;
+        double v;
+        if (spd) {
+            const int64_t hi = r > c ? r : c, lo = r > c ? c : r;
+            v = u01(seed, (uint64_t)(hi * cols + lo));
+            if (r == c) v = v + alpha;
+        } else {
+            v = u01(seed, (uint64_t)(r * cols + c));
+        }
+        out[e] = (T)v;
+    }
+}
+
+int gen_tile(uint64_t seed, int64_t rows, int64_t cols, int dtype, int b, int64_t ti, int64_t tj, int spd, void *out,
+             cudaStream_t s)
+{
+    (void)rows;
+    const double alpha = cols >= 256 ? 2.5 * std::sqrt((double)cols) : (double)cols;  // reading R8 (n = cols)
+    const int grid = 148 * 4;
+    count_launch();
+    if (dtype == 0) gen_tile_kernel<float><<<grid, 256, 0, s>>>(seed, cols, b, ti, tj, spd, alpha, (float *)out);
+    else if (dtype == 1) gen_tile_kernel<double><<<grid, 256, 0, s>>>(seed, cols, b, ti, tj, spd, alpha, (double *)out);
+    else return -1;
+    return 0;
+}
+
+}  // namespace vsk

@@ -35,5 +35,7 @@ int builtin_elem_bytes(int version);
 int gen_uniform(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b, void *out,
                 cudaStream_t s);
 int gen_spd(uint64_t seed, int64_t n, int dtype, int tile_b, void *out, cudaStream_t s);
+int gen_tile(uint64_t seed, int64_t rows, int64_t cols, int dtype, int b, int64_t ti, int64_t tj, int spd, void *out,
+             cudaStream_t s);
 
 }  // namespace vsk

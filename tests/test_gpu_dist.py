@@ -1,0 +1,111 @@
+"""One process per GPU (§8(e)) on the GPU: a 2-rank job (both ranks on cuda:0 when only one
+device is present — CUDA IPC works between processes on one device) runs the sharded tiled
+matmul + tiled Cholesky with owner computes, NVLink/IPC tile pulls and cross-rank
+completion tags; every rank checks the tiles it owns against the CPU oracle."""
+import os
+import socket
+
+import numpy as np
+import pytest
+
+pytestmark = pytest.mark.gpu
+
+MM_N, MM_B, CH_N, CH_B = 1024, 256, 2048, 256
+
+
+def _port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+def _worker(rank, world, port, q):
+    import torch
+    import torch.distributed as dist
+
+    import bench
+    import oracle
+    import paper_conf_ipps_planasbal13_b200 as vs
+    import vsgen
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        torch.cuda.set_device(rank % torch.cuda.device_count())
+
+        def gather(obj):
+            out = [None] * world
+            dist.all_gather_object(out, obj)
+            return out
+
+        rt = vs.Runtime(vs.vs_config_default(lam=1, slots_per_gpu=2, priority=1))
+        shm = gather("/vsched_test_%d" % os.getpid() if rank == 0 else None)[0]
+        if rank == 0:
+            rt.vs_dist_init(rank, world, shm)
+        dist.barrier()
+        if rank != 0:
+            rt.vs_dist_init(rank, world, shm)
+        dist.barrier()
+        wl = bench.Workload(rt, MM_N, MM_B, CH_N, CH_B, rank=rank, nranks=world, gather=gather)
+        for _ in range(2):                       # second step re-runs on learned tables
+            wl.step(dist.barrier)
+        dist.barrier()
+        torch.cuda.synchronize()
+        # ---- matmul: owned C tiles vs oracle
+        A = vsgen.uniform(bench.SEED_MM, MM_N, MM_N)
+        B = vsgen.uniform(bench.SEED_MM + 1000, MM_N, MM_N)
+        Cref = oracle.matmul(A, B)
+        nt = MM_N // MM_B
+        own = [(i, j) for i in range(nt) for j in range(nt) if bench.tile_owner(i, j, world) == rank]
+        Cown = wl.C.cpu().numpy()
+        err_mm = max(oracle.relF(Cown[k], Cref[i * MM_B:(i + 1) * MM_B, j * MM_B:(j + 1) * MM_B])
+                     for k, (i, j) in enumerate(own))
+        # ---- Cholesky: owned L tiles vs oracle
+        S = vsgen.spd(bench.SEED_CH, CH_N)
+        L, info = oracle.cholesky(S)
+        ntc = CH_N // CH_B
+        ownc = [(i, j) for i in range(ntc) for j in range(i + 1) if bench.tile_owner(i, j, world) == rank]
+        Sown = wl.S.cpu().numpy()
+        err_ch = 0.0
+        for k, (i, j) in enumerate(ownc):
+            got = Sown[k]
+            ref = L[i * CH_B:(i + 1) * CH_B, j * CH_B:(j + 1) * CH_B]
+            if i == j:
+                got, ref = np.tril(got), np.tril(ref)
+            err_ch = max(err_ch, oracle.relF(got, ref))
+        st = rt.vs_stats()
+        q.put((rank, err_mm, err_ch, len(own), len(ownc), st.tasks_completed, st.device_tx_bytes, st.tracker, info))
+        dist.barrier()
+        rt.close()
+    except Exception as e:   # report instead of hanging the parent
+        q.put((rank, "error", repr(e)))
+        raise
+    finally:
+        dist.destroy_process_group()
+
+
+def test_two_ranks_sharded_matmul_cholesky(gpu):
+    import torch.multiprocessing as mp
+    world = 2
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _port()
+    procs = [ctx.Process(target=_worker, args=(r, world, port, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    res = [q.get(timeout=600) for _ in range(world)]
+    for p in procs:
+        p.join(timeout=120)
+    for r in res:
+        assert r[1] != "error", r
+        rank, err_mm, err_ch, n_mm, n_ch, completed, dtx, tracker, info = r
+        assert info == 0
+        assert n_mm > 0 and n_ch > 0
+        assert err_mm <= 1e-5, (rank, err_mm)
+        assert err_ch <= 1e-5, (rank, err_ch)
+        assert tracker == 1                      # completion words are used across ranks
+        assert dtx > 0                           # remote tiles were pulled
+    for p in procs:
+        assert p.exitcode == 0
