@@ -81,9 +81,16 @@ struct TcEngine {
     {
         return tc::tc_gemm<NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s, ctx);
     }
+    // Recursive: X1 = X1 L11^{-T}; X2 -= X1 L21^T (one large tcgen05 GEMM); X2 = X2 L22^{-T};
+    // column blocks of at most 256 are solved by the fused single-launch tc_trsm kernel.
     static int trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
     {
-        return tc::tc_trsm(rows, n, L, ldl, X, ldx, s, ctx);
+        if (n <= 256) return tc::tc_trsm(rows, n, L, ldl, X, ldx, s, ctx);
+        const int h = (n / 2) / 64 * 64, r = n - h;
+        int rc = trsm(rows, h, L, ldl, X, ldx, s, ctx);
+        if (!rc) rc = gemm<true, true, false>(rows, r, h, X, ldx, L + (int64_t)h * ldl, ldl, X + h, ldx, s, ctx);
+        if (!rc) rc = trsm(rows, r, L + (int64_t)h * ldl + h, ldl, X + h, ldx, s, ctx);
+        return rc;
     }
 };
 
