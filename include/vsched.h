@@ -121,6 +121,11 @@ typedef struct {
                           GEMM_NT < MATMUL < user types, and POTRF/TRSM/SYRK launched on a
                           high-priority stream of their worker (L711-718: potrf must run as
                           soon as it is ready) */
+    int group_ratio_permille; /* 0: DataSetSize groups match exactly (R20).  r > 0: a new size
+                          joins the first group of its type (creation order) within a factor
+                          1 + r/1000 (range groups, future work L984-993; NEXT-3) */
+    int ewma_weight;   /* 0: ExecTime is the arithmetic mean (L408-411).  w in 1..1024: recency-
+                          weighted mean m += (x - m) * w / 1024 (footnote 3, L458-460; NEXT-3) */
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,

@@ -39,7 +39,8 @@ ERRORS = {0: "VS_OK", -1: "VS_E_INVAL", -2: "VS_E_NOMEM", -3: "VS_E_CUDA", -4: "
 class vs_config(Structure):
     _fields_ = [("exec", c_int), ("n_gpus", c_int), ("device_base", c_int), ("slots_per_gpu", c_int),
                 ("lambda_", c_int), ("policy", c_int), ("fixed_version", c_int), ("learning", c_int),
-                ("mode", c_int), ("replay", c_int), ("flush", c_int), ("lookahead", c_int), ("priority", c_int)]
+                ("mode", c_int), ("replay", c_int), ("flush", c_int), ("lookahead", c_int), ("priority", c_int),
+                ("group_ratio_permille", c_int), ("ewma_weight", c_int)]
 
 
 class vs_stats_t(Structure):

@@ -226,3 +226,37 @@ def test_rr_learning_variant_keeps_cycling():
     log = rt.vs_decision_log()
     # all 12 are ready at t=0, no time has been recorded yet: paper-literal RR alternates
     assert [r[1] for r in log] == [0, 1] * 6
+
+
+@pytest.mark.parametrize("ratio,ewma", [(0, 0), (300, 0), (300, 256), (0, 512)])
+def test_next3_range_groups_and_ewma_match_model(ratio, ewma):
+    # NEXT-3: range groups (L984-993) + recency-weighted mean (fn. 3, L458-460), C++ vs O3.
+    sizes = [128, 144, 160, 192, 256, 320]
+    rt = vs.Runtime(vs.vs_config_default(exec=vs.VS_EXEC_SIM, n_gpus=1, slots_per_gpu=2, lam=2,
+                                         group_ratio_permille=ratio, ewma_weight=ewma))
+    t = rt.vs_type_create("MATMUL", [vs.VS_IN, vs.VS_IN, vs.VS_INOUT])
+    rt.vs_version_add(t, "a", ALL)
+    rt.vs_version_add(t, "b", ALL)
+    m = SchedModel(1, 2, 2, group_ratio=ratio, ewma=ewma)
+    mt = m.add_type("MATMUL", [("a", ALL), ("b", ALL)])
+    k = 0
+    dur = lambda ty, nb, v: (nb // 1000) * (3 if v == 0 else 2) + 100 * v   # noqa: E731
+    for rep in range(6):
+        for b in sizes:
+            nb = b * b * 4
+            ids = [rt.vs_data_register(0x10000000 + k + i * nb, 0, nb) for i in range(3)]
+            mids = [m.add_data(nb) for _ in range(3)]
+            k += 3 * nb
+            rt.vs_submit(t, ids)
+            m.submit(mt, [(mids[0], "in"), (mids[1], "in"), (mids[2], "inout")])
+    for b in sizes:
+        for v in range(2):
+            rt.vs_replay_set(t, 3 * b * b * 4, v, dur(t, 3 * b * b * 4, v))
+    rt.vs_wait_all()
+    ref = m.simulate(dur)
+    got = rt.vs_decision_log()
+    assert [r[:4] for r in got] == [r[:4] for r in ref]
+    ngroups = len(rt.vs_group_stats())
+    assert ngroups == (len(sizes) if ratio == 0 else len({id(g) for g in m.groups.values()}))
+    if ratio:
+        assert ngroups < len(sizes)
