@@ -126,6 +126,9 @@ typedef struct {
                           1 + r/1000 (range groups, future work L984-993; NEXT-3) */
     int ewma_weight;   /* 0: ExecTime is the arithmetic mean (L408-411).  w in 1..1024: recency-
                           weighted mean m += (x - m) * w / 1024 (footnote 3, L458-460; NEXT-3) */
+    int locality_gbps; /* 0: earliest executor ignores data placement (paper).  g > 0: add
+                          (bytes of the task not yet on the worker's GPU) / g GB/s to EFT
+                          (locality-aware versioning, future work L978-984; NEXT-1) */
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,

@@ -260,3 +260,38 @@ def test_next3_range_groups_and_ewma_match_model(ratio, ewma):
     assert ngroups == (len(sizes) if ratio == 0 else len({id(g) for g in m.groups.values()}))
     if ratio:
         assert ngroups < len(sizes)
+
+
+def _locality_run(gbps):
+    # NEXT-1 (L978-984): EFT + bytes not on the worker's GPU / bandwidth; 2 GPUs x 2 slots.
+    nt, b = 4, 256
+    nbytes = b * b * 4
+    rt = vs.Runtime(vs.vs_config_default(exec=vs.VS_EXEC_SIM, n_gpus=2, slots_per_gpu=2, lam=1,
+                                         locality_gbps=gbps))
+    t = rt.vs_type_create("MATMUL", [vs.VS_IN, vs.VS_IN, vs.VS_INOUT])
+    rt.vs_version_add(t, "a", ALL)
+    rt.vs_version_add(t, "b", ALL)
+    ids = [rt.vs_data_register(_fake_ptr(i, nbytes), i % 2, nbytes) for i in range(3 * nt * nt)]
+    rt.vs_app_matmul(t, nt, nt, nt, ids[:16], ids[16:32], ids[32:])
+    rt.vs_replay_set(t, 3 * nbytes, 0, 30000)
+    rt.vs_replay_set(t, 3 * nbytes, 1, 20000)
+    m = SchedModel(2, 2, 1, locality_gbps=gbps)
+    mt = m.add_type("MATMUL", [("a", ALL), ("b", ALL)])
+    mids = [m.add_data(nbytes, home=i % 2) for i in range(3 * nt * nt)]
+    submit_matmul(m, mt, nt, nt, nt, mids[:16], mids[16:32], mids[32:])
+    rt.vs_wait_all()
+    ref = m.simulate(lambda ty, nb, v: [30000, 20000][v])
+    got = rt.vs_decision_log()
+    assert [r[:4] for r in got] == [r[:4] for r in ref]
+    # chain migrations: consecutive tasks of one C tile on different GPUs
+    gpu_of = {r[0]: r[2] // 2 for r in got}
+    return sum(gpu_of[c * nt + k] != gpu_of[c * nt + k - 1] for c in range(nt * nt) for k in range(1, nt))
+
+
+@pytest.mark.parametrize("gbps", [0, 50])
+def test_next1_locality_eft_matches_model(gbps):
+    _locality_run(gbps)
+
+
+def test_next1_locality_reduces_migrations():
+    assert _locality_run(50) <= _locality_run(0)
