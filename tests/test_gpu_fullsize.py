@@ -29,19 +29,30 @@ def test_fullsize_bench_configuration(gpu):
     for r in rows:
         a = vsgen.uniform_idx(bench.SEED_MM, np.arange(r * N, (r + 1) * N, dtype=np.uint64)).astype(np.float32)
         ref = oracle.matmul(a[None, :], Bfull)[0]
-        got = wl.C[r // b, :, r % b, :].reshape(-1).cpu().numpy()
+        got = wl.C.view(nt, nt, b, b)[r // b, :, r % b, :].reshape(-1).cpu().numpy()
         assert oracle.relF(got, ref) <= 1e-5, r
     # Freivalds on the whole product: A (B x) vs C x
     rng = np.random.default_rng(1)
     x = rng.standard_normal(N)
     Afull = vsgen.uniform(bench.SEED_MM, N, N)
-    C = vsgen.from_tiles(wl.C.cpu().numpy()).astype(np.float64)
+    C = vsgen.from_tiles(wl.C.view(nt, nt, b, b).cpu().numpy()).astype(np.float64)
     lhs = Afull.astype(np.float64) @ (Bfull.astype(np.float64) @ x)
     assert np.linalg.norm(lhs - C @ x) / np.linalg.norm(lhs) <= 1e-5
     del C, Afull, Bfull
     # ---- Cholesky: leading 2048 block vs oracle; residual on the full matrix
     Nc, bc = bench.CH_N, bench.CH_B
-    L = np.tril(vsgen.from_tiles(wl.S.cpu().numpy()))
+    ntc = Nc // bc
+
+    def full(T):      # lower tiles (i, j <= i) in row order -> dense lower matrix
+        out = np.zeros((Nc, Nc), np.float32)
+        host = T.cpu().numpy()
+        k = 0
+        for i in range(ntc):
+            for j in range(i + 1):
+                out[i * bc:(i + 1) * bc, j * bc:(j + 1) * bc] = host[k]
+                k += 1
+        return out
+    L = np.tril(full(wl.S))
     k = 2048
     r = np.arange(k, dtype=np.uint64)[:, None]
     c = np.arange(k, dtype=np.uint64)[None, :]
@@ -52,7 +63,7 @@ def test_fullsize_bench_configuration(gpu):
     lo, slo = np.tril_indices(k), np.tril_indices(k, -1)
     assert oracle.relF(L[:k, :k][lo], Lk[lo]) <= 1e-5
     assert oracle.relF(L[:k, :k][slo], Lk[slo]) <= 1e-5
-    A = vsgen.from_tiles(wl.S0.cpu().numpy())
+    A = full(wl.S0)
     A = np.tril(A) + np.tril(A, -1).T
     x = rng.standard_normal(Nc)
     Ax = A.astype(np.float64) @ x

@@ -42,7 +42,7 @@ def worker(rank, world, port, what, deadline):
         dist.all_gather_object(out, obj)
         return out
 
-    rt = vs.Runtime(vs.vs_config_default(lam=1, slots_per_gpu=2, priority=0))
+    rt = vs.Runtime(vs.vs_config_default(lam=1, slots_per_gpu=2, priority=int(os.environ.get("DBG_PRIO", "0"))))
     shm = gather("/vsched_dbg_%d" % os.getpid() if rank == 0 else None)[0]
     if rank == 0:
         rt.vs_dist_init(rank, world, shm)
@@ -51,7 +51,8 @@ def worker(rank, world, port, what, deadline):
         rt.vs_dist_init(rank, world, shm)
     dist.barrier()
     log("dist_init ok", shm)
-    wl = bench.Workload(rt, 512, 256, 1024, 256, rank=rank, nranks=world, gather=gather,
+    sz = [int(x) for x in os.environ.get("DBG_SIZES", "512,256,1024,256").split(",")]
+    wl = bench.Workload(rt, sz[0], sz[1], sz[2], sz[3], rank=rank, nranks=world, gather=gather,
                         with_mm=what in ("mm", "both"), with_ch=what in ("ch", "both"))
     log("workload ok")
     for s in range(2):
