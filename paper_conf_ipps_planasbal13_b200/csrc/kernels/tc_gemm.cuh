@@ -191,7 +191,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
 
     if (threadIdx.x == 0) {
         for (int s = 0; s < STAGES; s++) {
-            mbar_init(&full[s], NPROD);
+            mbar_init(&full[s], NPROD / 32);   // one arrive per producer warp
             mbar_init(&empty[s], 1);
         }
         mbar_init(acc_full, 1);
@@ -276,7 +276,8 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                 }
             }
             fence_proxy_async();
-            mbar_arrive(&full[s]);
+            __syncwarp();                            // the warp's stores + fences precede...
+            if (lane == 0) mbar_arrive(&full[s]);    // ...one release-arrive per warp
         };
         // two k-blocks of loads in flight (register double buffer, loop unrolled by 2)
         float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];

@@ -109,7 +109,7 @@ tc_gemm2_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const
 
     if (threadIdx.x == 0) {
         for (int s = 0; s < STAGES2; s++) {
-            mbar_init(&full[s], 2 * NPROD);    // both CTAs' producers arrive on the leader's
+            mbar_init(&full[s], 2 * NPROD / 32);   // one arrive per producer warp of both CTAs
             mbar_init(&empty[s], 1);
         }
         mbar_init(acc_full, 1);
@@ -181,7 +181,8 @@ tc_gemm2_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const
                 }
             }
             fence_proxy_async();
-            mbar_arrive_cluster(&full[s], 0);      // the leader's barrier
+            __syncwarp();
+            if (lane == 0) mbar_arrive_cluster(&full[s], 0);      // the leader's barrier, one per warp
         };
         float4 ra0[APER2], rb0[BPER2], ra1[APER2], rb1[BPER2];
         load(ra0, rb0, 0);

@@ -75,7 +75,7 @@ tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, 
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     if (threadIdx.x == 0) {
         for (int s = 0; s < STAGES; s++) {
-            mbar_init(&full[s], NPROD);
+            mbar_init(&full[s], NPROD / 32);
             mbar_init(&empty[s], 1);
         }
         mbar_init(acc_full, 1);
@@ -148,7 +148,8 @@ tc_trsm_kernel(int rows, int n, const float *__restrict__ L, int ldl, float *X, 
                     store_split(b_big, b_small, kmaj_off(row, c), rb[p]);
                 }
                 fence_proxy_async();
-                mbar_arrive(&full[s]);
+                __syncwarp();
+                if (lane == 0) mbar_arrive(&full[s]);   // one release-arrive per producer warp
                 gkb++;
             };
             if (nk > 0) {
