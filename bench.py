@@ -34,6 +34,9 @@ sys.path.insert(0, ROOT)
 MM_N, MM_B = 16384, 1024
 CH_N, CH_B = 32768, 1024
 SEED_MM, SEED_CH = 3, 4
+# runtime configuration the bench times (env VS_SLOTS / VS_PRIORITY / VS_QDEPTH override):
+# lambda 3, 6 workers (streams) per GPU, NEXT-4 bottom-level priority with queue depth 2
+RT_DEFAULTS = dict(lam=3, slots=6, priority=2, qdepth=2)
 F32_VERSIONS_MASK = 0b111     # simt_f32 | tc_3xtf32 | f64in_f32io
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
@@ -327,8 +330,10 @@ def main():
     ap.add_argument("--steps", type=int, default=5)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
-    ap.add_argument("--slots", type=int, default=int(os.environ.get("VS_SLOTS", "4")))
-    ap.add_argument("--lam", type=int, default=3)
+    ap.add_argument("--slots", type=int, default=int(os.environ.get("VS_SLOTS", RT_DEFAULTS["slots"])))
+    ap.add_argument("--priority", type=int, default=int(os.environ.get("VS_PRIORITY", RT_DEFAULTS["priority"])))
+    ap.add_argument("--qdepth", type=int, default=int(os.environ.get("VS_QDEPTH", RT_DEFAULTS["qdepth"])))
+    ap.add_argument("--lam", type=int, default=RT_DEFAULTS["lam"])
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--small", action="store_true", help="cfg1/cfg2-sized smoke of the bench itself")
@@ -364,12 +369,12 @@ def main():
 
     mm_n, mm_b, ch_n, ch_b = (MM_N, MM_B, CH_N, CH_B) if not args.small else (1024, 256, 4096, 512)
     with_mm, with_ch = args.only in ("mm", "both"), args.only in ("ch", "both")
-    # critical-path priority (NEXT-4, vs_config.priority) is on by default in the bench;
-    # VS_PRIORITY=0 reproduces the paper-literal FIFO ready order (R15)
-    prio = int(os.environ.get("VS_PRIORITY", "1"))
+    # critical-path scheduling (NEXT-4: vs_config.priority / queue_depth) is on by default
+    # in the bench; --priority 0 --qdepth 0 reproduces the paper-literal rule (R15)
+    prio, qdepth = args.priority, args.qdepth
     look = int(os.environ.get("VS_LOOKAHEAD", "0"))
     cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0,
-                               priority=prio, lookahead=look)
+                               priority=prio, lookahead=look, queue_depth=qdepth)
     rt = vs.Runtime(cfg)
     if world > 1:
         shm = gather("/vsched_%d_%d" % (os.getpid(), int(time.time())) if rank == 0 else None)[0]
@@ -436,7 +441,7 @@ def main():
     # ---- e2e: same step through the C ABI with HOST (pinned) buffers, copies inside the timed region
     e2e = None
     if not args.no_e2e and world == 1:
-        rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look))
+        rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look, queue_depth=qdepth))
         wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, with_mm=with_mm, with_ch=with_ch)
         wl2.step()     # warm-up incl. learning
         tsum, h2d, d2h = 0.0, 0, 0
@@ -489,7 +494,7 @@ def main():
             "roofline": roof,
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
             "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
-            "runtime_options": {"lookahead": look, "priority": prio, "mode": "runahead"},
+            "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "mode": "runahead"},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
             "device_tx_bytes_per_step": int((st1.device_tx_bytes - st0.device_tx_bytes) / args.steps),

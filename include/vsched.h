@@ -120,7 +120,10 @@ typedef struct {
                           1: critical-path first (NEXT-4): ready order POTRF < TRSM < SYRK <
                           GEMM_NT < MATMUL < user types, and POTRF/TRSM/SYRK launched on a
                           high-priority stream of their worker (L711-718: potrf must run as
-                          soon as it is ready) */
+                          soon as it is ready);
+                          2: bottom level first (NEXT-4, generic): ready order by the
+                          longest path (in tasks) from the task to the end of the submitted
+                          DAG, larger first, ties by id; same high-priority streams as 1 */
     int group_ratio_permille; /* 0: DataSetSize groups match exactly (R20).  r > 0: a new size
                           joins the first group of its type (creation order) within a factor
                           1 + r/1000 (range groups, future work L984-993; NEXT-3) */
@@ -129,12 +132,18 @@ typedef struct {
     int locality_gbps; /* 0: earliest executor ignores data placement (paper).  g > 0: add
                           (bytes of the task not yet on the worker's GPU) / g GB/s to EFT
                           (locality-aware versioning, future work L978-984; NEXT-1) */
+    int queue_depth;   /* 0: a ready task is assigned at once to its earliest executor,
+                          whatever that worker's queue holds (paper, L414-422).  d > 0
+                          (run-ahead and SIM only): a ready task is assigned only while some
+                          worker holds fewer than d virtual tasks (running + queued), and only
+                          to such workers; the rest wait in the (priority) ready queue, so a
+                          task released later on the critical path overtakes them (NEXT-4) */
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,
  * run-ahead, live timing, flush.  Environment overrides applied by vs_create (L277-288):
  * VS_LAMBDA, VS_SLOTS, VS_POLICY(=versioning|fixed:<v>), VS_LEARNING(=hold|rr),
- * VS_MODE(=runahead|ready), VS_LOOKAHEAD(=n), VS_PRIORITY(=0|1). */
+ * VS_MODE(=runahead|ready), VS_LOOKAHEAD(=n), VS_PRIORITY(=0|1|2), VS_QDEPTH(=d). */
 void vs_config_default(vs_config *cfg);
 
 /* Create a runtime.  *out receives an opaque handle owning scheduler state, DAG,

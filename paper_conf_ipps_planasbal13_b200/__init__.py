@@ -40,7 +40,8 @@ class vs_config(Structure):
     _fields_ = [("exec", c_int), ("n_gpus", c_int), ("device_base", c_int), ("slots_per_gpu", c_int),
                 ("lambda_", c_int), ("policy", c_int), ("fixed_version", c_int), ("learning", c_int),
                 ("mode", c_int), ("replay", c_int), ("flush", c_int), ("lookahead", c_int), ("priority", c_int),
-                ("group_ratio_permille", c_int), ("ewma_weight", c_int), ("locality_gbps", c_int)]
+                ("group_ratio_permille", c_int), ("ewma_weight", c_int), ("locality_gbps", c_int),
+                ("queue_depth", c_int)]
 
 
 class vs_stats_t(Structure):

@@ -165,6 +165,22 @@ __device__ __forceinline__ void store_split(uint8_t *big, uint8_t *small, uint32
     *reinterpret_cast<float4 *>(small + off) = make_float4(v.x - b.x, v.y - b.y, v.z - b.z, v.w - b.w);
 }
 
+// NN B operand: producer thread t, unit p holds the 4 (k) x 4 (n) block at k-chunk kq,
+// n-quad nq.  Lane bits: [0] = nq bit 0, [1:2] = kq bits 0-1, [3:4] = nq bits 1-2; the
+// warp/unit index supplies kq bit 2 and the high nq bits.  A warp's LDG.128 then covers 4
+// k-rows x 128 contiguous bytes, and the 8 lanes of each STS.128 phase (rows 8m+i, 8m+4+i;
+// 4 consecutive k-chunks) land on 8 distinct swizzled chunks: conflict-free with the
+// transpose done in registers at compile-time indices.
+template <int BN>
+__device__ __forceinline__ void nn_unit(int t, int p, int &kq, int &nq)
+{
+    static_assert(BN >= 128 && BN % 32 == 0, "nn_unit needs >= 1 unit per producer thread");
+    constexpr int NG = BN / 32;
+    const int lane = t & 31, idx = (t >> 5) + p * (NPROD / 32);
+    kq = ((lane >> 1) & 3) | ((idx / NG) << 2);
+    nq = (lane & 1) | (((lane >> 3) & 3) << 1) | ((idx % NG) << 3);
+}
+
 template <int BN, bool NT, bool NEG, bool LOWER>
 __global__ void __launch_bounds__(NTHREADS, 1)
 tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const float *__restrict__ B, int ldb,
@@ -227,10 +243,11 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                     rb[p] = (n0 + row < N) ? __ldg(reinterpret_cast<const float4 *>(B + (int64_t)(n0 + row) * ldb + k0 + 4 * c)) : z4;
                 }
             } else {
-                // NN: 4 (k) x 4 (n) blocks; unit u -> kq = u / (BN/4), nq = u % (BN/4)
+                // NN: 4 (k) x 4 (n) blocks, see nn_unit
 #pragma unroll
                 for (int p = 0; p < BPER / 4; p++) {
-                    const int u = t + p * NPROD, kq = u / (BN / 4), nq = u % (BN / 4);
+                    int kq, nq;
+                    nn_unit<BN>(t, p, kq, nq);
                     const bool ok = n0 + 4 * nq < N;
 #pragma unroll
                     for (int i = 0; i < 4; i++)
@@ -258,21 +275,14 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
             } else {
 #pragma unroll
                 for (int p = 0; p < BPER / 4; p++) {
-                    const int u = t + p * NPROD, kq = u / (BN / 4), nq = u % (BN / 4);
+                    int kq, nq;
+                    nn_unit<BN>(t, p, kq, nq);
                     const float4 r0 = rb[4 * p], r1 = rb[4 * p + 1], r2 = rb[4 * p + 2], r3 = rb[4 * p + 3];
                     // column n' of the 4x4 block = K-major 16-byte chunk of row n = 4nq+n'
-                    // rotate which column each thread stores first so the 8 threads of an
-                    // STS.128 phase hit 8 distinct (row & 7) -> 8 distinct swizzled chunks
-                    const int rot = (nq >> 1) & 3;
-#pragma unroll
-                    for (int qq = 0; qq < 4; qq++) {
-                        const int i = (qq + rot) & 3;
-                        const float4 col = i == 0 ? make_float4(r0.x, r1.x, r2.x, r3.x)
-                                         : i == 1 ? make_float4(r0.y, r1.y, r2.y, r3.y)
-                                         : i == 2 ? make_float4(r0.z, r1.z, r2.z, r3.z)
-                                                  : make_float4(r0.w, r1.w, r2.w, r3.w);
-                        store_split(b_big, b_small, kmaj_off(4 * nq + i, kq), col);
-                    }
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 0, kq), make_float4(r0.x, r1.x, r2.x, r3.x));
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 1, kq), make_float4(r0.y, r1.y, r2.y, r3.y));
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 2, kq), make_float4(r0.z, r1.z, r2.z, r3.z));
+                    store_split(b_big, b_small, kmaj_off(4 * nq + 3, kq), make_float4(r0.w, r1.w, r2.w, r3.w));
                 }
             }
             fence_proxy_async();

@@ -23,9 +23,9 @@ def test_library_exports_every_header_symbol():
     assert "sm_100a" in vs.vs_build_info()
 
 
-def _sim(n_gpus=1, slots=4, lam=3, learning=vs.VS_LEARN_HOLD):
+def _sim(n_gpus=1, slots=4, lam=3, learning=vs.VS_LEARN_HOLD, **kw):
     return vs.Runtime(vs.vs_config_default(exec=vs.VS_EXEC_SIM, n_gpus=n_gpus, slots_per_gpu=slots, lam=lam,
-                                           learning=learning))
+                                           learning=learning, **kw))
 
 
 def _fake_ptr(i, nbytes):
@@ -295,3 +295,66 @@ def test_next1_locality_eft_matches_model(gbps):
 
 def test_next1_locality_reduces_migrations():
     assert _locality_run(50) <= _locality_run(0)
+
+
+# ---------------------------------------------------------------- NEXT-4 (R29)
+def _mixed(nt_mm, nt_ch, lam, slots, dur_us, n_gpus=1, model=True, **kw):
+    """Fig 1 matmul and the tiled Cholesky submitted to ONE runtime (the bench workload's
+    shape), replayed from a timing table; returns (C++ log, Python model log or None)."""
+    rt = _sim(n_gpus, slots, lam, **kw)
+    names = ("MATMUL", "POTRF", "TRSM", "SYRK", "GEMM_NT")
+    modes = ([vs.VS_IN, vs.VS_IN, vs.VS_INOUT], [vs.VS_INOUT], [vs.VS_IN, vs.VS_INOUT], [vs.VS_IN, vs.VS_INOUT],
+             [vs.VS_IN, vs.VS_IN, vs.VS_INOUT])
+    nbytes = 1024 * 1024 * 4
+    sizes = (3 * nbytes, nbytes, 2 * nbytes, 2 * nbytes, 3 * nbytes)
+    tys = []
+    for ti, (n, md) in enumerate(zip(names, modes)):
+        t = rt.vs_type_create(n, md)
+        for v in range(2):
+            rt.vs_version_add(t, "v%d" % v, ALL)
+            rt.vs_replay_set(t, sizes[ti], v, dur_us[ti] * 1000 * (3 if v == 0 else 1))
+        tys.append(t)
+    k = [0]
+
+    def reg():
+        k[0] += 1
+        return rt.vs_data_register(_fake_ptr(k[0], nbytes), 0, nbytes)
+    mm = [reg() for _ in range(3 * nt_mm * nt_mm)]
+    q = nt_mm * nt_mm
+    rt.vs_app_matmul(tys[0], nt_mm, nt_mm, nt_mm, mm[:q], mm[q:2 * q], mm[2 * q:])
+    A = {i * nt_ch + j: reg() for i in range(nt_ch) for j in range(i + 1)}
+    rt.vs_app_cholesky(tys, nt_ch, A)
+    rt.vs_wait_all()
+    got = rt.vs_decision_log()
+    rt.close()
+    if not model:
+        return got, None
+    m = SchedModel(n_gpus, slots, lam, priority=kw.get("priority", 0), qdepth=kw.get("queue_depth", 0))
+    mt = [m.add_type(n, [("v0", ALL), ("v1", ALL)]) for n in names]
+    mm_ = [m.add_data(nbytes) for _ in range(3 * q)]
+    submit_matmul(m, mt[0], nt_mm, nt_mm, nt_mm, mm_[:q], mm_[q:2 * q], mm_[2 * q:])
+    mA = {i * nt_ch + j: m.add_data(nbytes) for i in range(nt_ch) for j in range(i + 1)}
+    submit_cholesky(m, tuple(mt[1:]), nt_ch, mA)
+    idx = {t: i for i, t in enumerate(mt)}
+    ref = m.simulate(lambda ty, nb, v: dur_us[idx[ty]] * 1000 * (3 if v == 0 else 1))
+    return got, ref
+
+
+BENCH_US = (68, 1500, 330, 52, 50)   # measured per-task us at b=1024 (MATMUL POTRF TRSM SYRK GEMM_NT)
+
+
+@pytest.mark.parametrize("priority,qdepth,slots", [(0, 0, 4), (0, 2, 4), (2, 0, 3), (2, 1, 2), (2, 2, 6),
+                                                   (2, 3, 4)])
+def test_next4_priority_and_queue_depth_match_model(priority, qdepth, slots):
+    got, ref = _mixed(4, 6, 2, slots, BENCH_US, priority=priority, queue_depth=qdepth)
+    assert len(got) == len(ref) == 64 + 56
+    assert [r[:6] for r in got] == [r[:6] for r in ref]
+
+
+def test_next4_bottom_level_with_queue_depth_shortens_the_mixed_makespan():
+    # the bench workload's shape at 1/4 scale in each dimension; paper rule vs NEXT-4
+    span = {}
+    for key, kw in (("paper", {}), ("next4", dict(priority=2, queue_depth=2))):
+        got, _ = _mixed(8, 16, 3, 6, BENCH_US, model=False, **kw)
+        span[key] = max(r[5] for r in got)
+    assert span["next4"] < span["paper"]

@@ -1,6 +1,6 @@
 """Parity at BASELINE.json's full sizes, in the launch configuration bench.py times
-(cfg3 matmul N=16384 b=1024 + cfg4 Cholesky N=32768 b=1024, 4 slots, lambda=3, all f32
-versions, run-ahead): sampled outputs the oracle computes one by one, plus properties that
+(cfg3 matmul N=16384 b=1024 + cfg4 Cholesky N=32768 b=1024, bench.RT_DEFAULTS: lambda 3,
+6 slots, bottom-level priority, queue depth 2; all f32 versions, run-ahead): sampled outputs the oracle computes one by one, plus properties that
 hold at any size."""
 import numpy as np
 import pytest
@@ -16,7 +16,9 @@ def test_fullsize_bench_configuration(gpu):
     import torch
 
     import bench
-    rt = vs.Runtime(vs.vs_config_default(lam=3, slots_per_gpu=4))
+    d = bench.RT_DEFAULTS
+    rt = vs.Runtime(vs.vs_config_default(lam=d["lam"], slots_per_gpu=d["slots"], priority=d["priority"],
+                                         queue_depth=d["qdepth"]))
     wl = bench.Workload(rt)
     wl.step()          # learning happens here (cold)
     wl.step()          # warm step, as timed by bench.py

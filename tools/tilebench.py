@@ -63,11 +63,12 @@ def main():
     ap.add_argument("--streams", type=int, default=1)
     ap.add_argument("--types", default="0,1,2,3,4")
     ap.add_argument("--versions", default="0,1,2,3")
+    ap.add_argument("--iters", type=int, default=20)
     a = ap.parse_args()
     for ttype in map(int, a.types.split(",")):
         for version in map(int, a.versions.split(",")):
             for b in a.sizes:
-                us, gf = bench(ttype, version, b, a.streams)
+                us, gf = bench(ttype, version, b, a.streams, a.iters)
                 print(json.dumps({"type": vs.TYPE_NAMES[ttype], "version": vs.VERSION_NAMES[version], "b": b,
                                   "streams": a.streams, "us_per_task": round(us, 2), "gflops": round(gf, 1)}))
                 sys.stdout.flush()
