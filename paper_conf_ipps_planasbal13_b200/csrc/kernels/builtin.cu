@@ -5,21 +5,24 @@
 //
 //   version        storage  GEMM engine (matmul/gemm/syrk + potrf/trsm updates)   trsm
 //   simt_f32       fp32     simt_gemm<float,float>   (FFMA, bit-exact Fig 1 order)  blocked
-//   tc_3xtf32      fp32     tc_gemm (tcgen05/TMEM 3xTF32)                          tc_trsm (1 launch)
+//   tc_3xtf32      fp32     tc_gemm (tcgen05/TMEM 3xTF32)                          tc_panel (1 launch)
 //   f64in_f32io    fp32     dmma_gemm<float>  (DMMA on upcast operands)            blocked
 //   dfma_f64       fp64     simt_gemm<double,double> (DFMA)                        blocked
 //   dmma_f64       fp64     dmma_gemm<double>  (mma.sync f64)                      blocked
 //
-// potrf (all versions) is recursive: potrf(A11); A21 <- A21 L11^{-T} (trsm);
+// potrf of tc_3xtf32 is the single-launch left-looking tc_panel kernel (tc_panel.cuh).
+// potrf of the other versions is recursive: potrf(A11); A21 <- A21 L11^{-T} (trsm);
 // A22 -= A21 A21^T (lower GEMM); potrf(A22), down to an NB x NB diagonal block factored
 // in registers (simt_chol.cuh).  Blocked trsm: NB-wide panels solved by trsm_panel,
 // remaining columns updated by the engine's GEMM.
+#include <type_traits>
+
 #include "dmma_gemm.cuh"
 #include "kernels.hpp"
 #include "simt_chol.cuh"
 #include "simt_gemm.cuh"
 #include "tc_gemm.cuh"
-#include "tc_trsm.cuh"
+#include "tc_panel.cuh"
 
 #include "vsched.h"
 
@@ -81,16 +84,10 @@ struct TcEngine {
     {
         return tc::tc_gemm<NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s, ctx);
     }
-    // Recursive: X1 = X1 L11^{-T}; X2 -= X1 L21^T (one large tcgen05 GEMM); X2 = X2 L22^{-T};
-    // column blocks of at most 256 are solved by the fused single-launch tc_trsm kernel.
+    // single-launch left-looking panel kernel (tc_panel.cuh)
     static int trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
     {
-        if (n <= 256) return tc::tc_trsm(rows, n, L, ldl, X, ldx, s, ctx);
-        const int h = (n / 2) / 64 * 64, r = n - h;
-        int rc = trsm(rows, h, L, ldl, X, ldx, s, ctx);
-        if (!rc) rc = gemm<true, true, false>(rows, r, h, X, ldx, L + (int64_t)h * ldl, ldl, X + h, ldx, s, ctx);
-        if (!rc) rc = trsm(rows, r, L + (int64_t)h * ldl + h, ldl, X + h, ldx, s, ctx);
-        return rc;
+        return tc::tc_trsm(rows, n, L, ldl, X, ldx, s, ctx);
     }
 };
 
@@ -133,7 +130,10 @@ int run_family(int type, int b, void *const *p, int *info, cudaStream_t s, const
     case VS_T_TRSM:  // B <- B L^{-T}              (R5)
         return E::trsm(b, b, (const Tin *)p[0], b, (Tin *)p[1], b, s, ctx);
     case VS_T_POTRF:  // A = L L^T in place        (L697-699, R9)
-        return potrf_rec<Tin, E>((Tin *)p[0], b, b, 0, info, s, ctx);
+        if constexpr (std::is_same<E, TcEngine>::value)
+            return tc::tc_potrf(b, (float *)p[0], b, 0, info, s, ctx);   // single launch (tc_panel.cuh)
+        else
+            return potrf_rec<Tin, E>((Tin *)p[0], b, b, 0, info, s, ctx);
     }
     return -1;
 }

@@ -158,11 +158,16 @@ __device__ __forceinline__ float4 split_big(float4 v)
 {
     return make_float4(to_tf32(v.x), to_tf32(v.y), to_tf32(v.z), to_tf32(v.w));
 }
+__device__ __forceinline__ void sts128(uint32_t addr, float4 v)
+{
+    asm volatile("st.shared.v4.f32 [%0], {%1,%2,%3,%4};" ::"r"(addr), "f"(v.x), "f"(v.y), "f"(v.z), "f"(v.w)
+                 : "memory");
+}
 __device__ __forceinline__ void store_split(uint8_t *big, uint8_t *small, uint32_t off, float4 v)
 {
     const float4 b = split_big(v);
-    *reinterpret_cast<float4 *>(big + off) = b;
-    *reinterpret_cast<float4 *>(small + off) = make_float4(v.x - b.x, v.y - b.y, v.z - b.z, v.w - b.w);
+    sts128(smem_u32(big) + off, b);
+    sts128(smem_u32(small) + off, make_float4(v.x - b.x, v.y - b.y, v.z - b.z, v.w - b.w));
 }
 
 // NN B operand: producer thread t, unit p holds the 4 (k) x 4 (n) block at k-chunk kq,
@@ -190,7 +195,8 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     using G = Cfg<BN>;
     constexpr int STAGES = G::STAGES;
     extern __shared__ uint8_t smem_raw[];
-    uint8_t *smem = (uint8_t *)(((uintptr_t)smem_raw + 1023) & ~(uintptr_t)1023);
+    // 1024-byte aligned, indexed from the __shared__ array so accesses stay LDS/STS
+    uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     uint64_t *full = (uint64_t *)(smem + STAGES * G::STAGE);
     uint64_t *empty = full + STAGES;
     uint64_t *acc_full = empty + STAGES;

@@ -89,7 +89,8 @@ tc_gemm2_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const
 {
     ctx_begin(ctx);
     extern __shared__ uint8_t smem_raw[];
-    uint8_t *smem = (uint8_t *)(((uintptr_t)smem_raw + 1023) & ~(uintptr_t)1023);
+    // 1024-byte aligned, indexed from the __shared__ array so accesses stay LDS/STS
+    uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     uint64_t *full = (uint64_t *)(smem + STAGES2 * STAGE2);
     uint64_t *empty = full + STAGES2;
     uint64_t *acc_full = empty + STAGES2;

@@ -1,0 +1,523 @@
+// tc_panel.cuh — single-launch tcgen05 3xTF32 left-looking panel kernel: the trsm task and
+// the potrf task of the tc_3xtf32 version (reading R5; PAPER.md L697-699 for the
+// algorithm of Cholesky, R9 for info).
+//
+//   TRSM:  X L^T = B (right side, L lower, transposed, non-unit), X overwrites B;
+//          rows x n block X (ldx), n x n lower L (ldl).
+//   POTRF: A = L L^T in place (n x n, lower triangle read and written, the strict upper
+//          triangle untouched, R7); first non-positive pivot -> *info = k_base + col + 1.
+// n a multiple of 64.  Each CTA owns 128 rows (TMEM lanes = rows) and walks the column
+// panels J (P = 128 wide, the last one possibly 64) left to right:
+//   1. T_J = B[:, J] - X[:, <J] L[J, <J]^T     (POTRF: A[:, J] - L[:, <J] L[J, <J]^T)
+//      tcgen05 3xTF32 MMA, M = 128, N = 128, K = 128 J, into one of two TMEM
+//      accumulators (panel parity) so that the MMA of panel J+1 runs while panel J is
+//      being solved.  A operand = the CTA's own solved columns, B operand = the panel's
+//      L rows; the k-blocks that need the columns solved in panel J wait for that panel
+//      only (mbarrier xdone).
+//   2. epilogue warps, one row each, per 16-column sub-block sb (compact code: a 16 x 16
+//      step is the only unrolled unit):
+//        x = b - acc[sb]  (b = the tile's current values, prefetched one sub-block ahead);
+//        TRSM / POTRF below the diagonal: forward substitution against L_JJ staged
+//          (transposed) in shared memory (x_c = t_c / l_cc; t_j -= x_c l_jc);
+//        POTRF diagonal CTA (CTA J holds panel J's diagonal block): right-looking
+//          factorisation column by column, the pivot row publishes l_cc = sqrt(t_c),
+//          every lower row scales and publishes l_ic (two named barriers per column);
+//        store x; acc[t] += x L[t, sb]^T for the later sub-blocks t (tcgen05.ld/st).
+// Roles: warps 0-3 producers (LDG -> split big/small -> 128B-swizzled K-major smem); warp 0
+// also allocates TMEM and, once all four producer warps filled a stage, issues its MMAs;
+// warps 4-7 epilogue (TMEM lane quarter = warp % 4).
+// POTRF: the other CTAs wait, through a per-launch progress word per CTA (release /
+// acquire at gpu scope), for CTA J to have finished panels < J before loading panel J's
+// L rows as MMA operand, and panel J before staging L_JJ.  Every CTA only waits on
+// lower-numbered CTAs of the same grid, which never wait on it: each one eventually
+// becomes resident and the launch cannot deadlock.
+// Division: rcp.approx + one Newton step (correctly rounded when the quotient is
+// representable: integer problems stay exact); sqrt is IEEE.
+#pragma once
+#include <atomic>
+#include <cstdlib>
+
+#include "tc_gemm.cuh"
+
+namespace vsk {
+namespace tc {
+
+constexpr int PNL = 128;   // panel width (= BM: panel J's diagonal block is CTA J's rows)
+constexpr int PSB = 16;    // solve sub-block
+constexpr int kFlagSlots = 4096;
+constexpr int kFlagCtas = 32;   // n <= 4096 -> at most 32 CTAs per potrf launch
+constexpr int PTHREADS = 256;   // 4 producer warps (warp 0 also issues the MMAs) + 4 epilogue
+                                // warps: 8 warps keep the 255-register budget (9 would cap at 168)
+
+struct PanelCfg {
+    static constexpr int STAGES = 2;
+    static constexpr int NP = 128;                          // producer threads
+    static constexpr int A_BYTES = BM * BK * 4;             // 16 KB
+    static constexpr int B_BYTES = PNL * BK * 4;            // 16 KB
+    static constexpr int STAGE = 2 * A_BYTES + 2 * B_BYTES; // 64 KB
+    static constexpr int LD = PNL + 4;                      // Lt row stride (16-byte rows)
+    static constexpr int LT_BYTES = PNL * LD * 4;           // 66 KB
+    static constexpr int SMEM = STAGES * STAGE + LT_BYTES + 1024 + 256;
+    static constexpr int APER = BM * BK / 4 / NP;           // 8
+    static constexpr int BPER = PNL * BK / 4 / NP;          // 8
+};
+
+// progress words of the potrf launches: slot = launch id % kFlagSlots, value =
+// (launch id << 8) | panels completed; ids grow, so no reset is needed between launches
+__device__ unsigned long long g_panel_flags[kFlagSlots][kFlagCtas];
+
+__device__ __forceinline__ float rcp_approx(float x)
+{
+    float r;
+    asm("rcp.approx.ftz.f32 %0, %1;" : "=f"(r) : "f"(x));
+    return r;
+}
+// t / l: x0 = t r, one Newton correction x = x0 + (t - x0 l) r
+__device__ __forceinline__ float div_nr(float t, float l, float r)
+{
+    const float x0 = t * r;
+    return fmaf(fmaf(-x0, l, t), r, x0);
+}
+// L2-coherent loads (data written by this or other CTAs during the launch)
+__device__ __forceinline__ float4 ld_f4_cg(const float *p)
+{
+    float4 v;
+    asm volatile("ld.global.cg.v4.f32 {%0,%1,%2,%3}, [%4];" : "=f"(v.x), "=f"(v.y), "=f"(v.z), "=f"(v.w) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ float ld_f_cg(const float *p)
+{
+    float v;
+    asm volatile("ld.global.cg.f32 %0, [%1];" : "=f"(v) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ unsigned long long ld_acquire(const unsigned long long *p)
+{
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ void st_release(unsigned long long *p, unsigned long long v)
+{
+    asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ void wait_flag(const unsigned long long *p, unsigned long long need)
+{
+    while (ld_acquire(p) < need) __nanosleep(64);
+}
+
+__device__ __forceinline__ void tmem_ld16(uint32_t taddr, float (&v)[16])
+{
+    uint32_t r[16];
+    asm volatile(
+        "tcgen05.ld.sync.aligned.32x32b.x16.b32 {%0,%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15}, [%16];"
+        : "=r"(r[0]), "=r"(r[1]), "=r"(r[2]), "=r"(r[3]), "=r"(r[4]), "=r"(r[5]), "=r"(r[6]), "=r"(r[7]),
+          "=r"(r[8]), "=r"(r[9]), "=r"(r[10]), "=r"(r[11]), "=r"(r[12]), "=r"(r[13]), "=r"(r[14]), "=r"(r[15])
+        : "r"(taddr));
+    asm volatile("tcgen05.wait::ld.sync.aligned;" ::: "memory");
+#pragma unroll
+    for (int i = 0; i < 16; i++) v[i] = __uint_as_float(r[i]);
+}
+__device__ __forceinline__ void tmem_st16(uint32_t taddr, const float (&v)[16])
+{
+    asm volatile(
+        "tcgen05.st.sync.aligned.32x32b.x16.b32 [%0], {%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,%16};" ::"r"(
+            taddr),
+        "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(v[4]), "f"(v[5]), "f"(v[6]), "f"(v[7]), "f"(v[8]), "f"(v[9]),
+        "f"(v[10]), "f"(v[11]), "f"(v[12]), "f"(v[13]), "f"(v[14]), "f"(v[15])
+        : "memory");
+    asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
+}
+// split-phase TMEM access for software pipelining: the wait takes the destination
+// registers as in/out operands so that no use of them is scheduled before it
+__device__ __forceinline__ void tmem_ld16_issue(uint32_t taddr, float (&v)[16])
+{
+    asm volatile(
+        "tcgen05.ld.sync.aligned.32x32b.x16.b32 {%0,%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15}, [%16];"
+        : "=f"(v[0]), "=f"(v[1]), "=f"(v[2]), "=f"(v[3]), "=f"(v[4]), "=f"(v[5]), "=f"(v[6]), "=f"(v[7]),
+          "=f"(v[8]), "=f"(v[9]), "=f"(v[10]), "=f"(v[11]), "=f"(v[12]), "=f"(v[13]), "=f"(v[14]), "=f"(v[15])
+        : "r"(taddr));
+}
+__device__ __forceinline__ void tmem_wait_ld(float (&v)[16])
+{
+    asm volatile("tcgen05.wait::ld.sync.aligned;"
+                 : "+f"(v[0]), "+f"(v[1]), "+f"(v[2]), "+f"(v[3]), "+f"(v[4]), "+f"(v[5]), "+f"(v[6]), "+f"(v[7]),
+                   "+f"(v[8]), "+f"(v[9]), "+f"(v[10]), "+f"(v[11]), "+f"(v[12]), "+f"(v[13]), "+f"(v[14]), "+f"(v[15])
+                 :
+                 : "memory");
+}
+__device__ __forceinline__ void tmem_st16_issue(uint32_t taddr, const float (&v)[16])
+{
+    asm volatile(
+        "tcgen05.st.sync.aligned.32x32b.x16.b32 [%0], {%1,%2,%3,%4,%5,%6,%7,%8,%9,%10,%11,%12,%13,%14,%15,%16};" ::"r"(
+            taddr),
+        "f"(v[0]), "f"(v[1]), "f"(v[2]), "f"(v[3]), "f"(v[4]), "f"(v[5]), "f"(v[6]), "f"(v[7]), "f"(v[8]), "f"(v[9]),
+        "f"(v[10]), "f"(v[11]), "f"(v[12]), "f"(v[13]), "f"(v[14]), "f"(v[15])
+        : "memory");
+}
+__device__ __forceinline__ void tmem_wait_st() { asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory"); }
+__device__ __forceinline__ void bar_epi() { asm volatile("bar.sync 2, 128;" ::: "memory"); }
+
+template <bool POTRF>
+__global__ void __launch_bounds__(PTHREADS, 1)
+tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int k_base, int *info,
+                unsigned long long launch_id, int overlap, TaskCtx ctx)
+{
+    ctx_begin(ctx);
+    using G = PanelCfg;
+    constexpr int P = PNL, STAGES = G::STAGES, LD = G::LD, NP = G::NP;
+    extern __shared__ uint8_t smem_raw[];
+    // 1024-byte aligned, indexed from the __shared__ array so accesses stay LDS/STS
+    uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
+    float *Lt = reinterpret_cast<float *>(smem + STAGES * G::STAGE);   // Lt[c * LD + j] = L_JJ[j][c]
+    __shared__ float Lr[P];       // reciprocals of the diagonal of L_JJ
+    __shared__ float colbuf[BM];  // POTRF diagonal CTA: published column
+    __shared__ float pivot;
+    uint64_t *full = (uint64_t *)((uint8_t *)Lt + G::LT_BYTES);
+    uint64_t *empty = full + STAGES;
+    uint64_t *accf = empty + STAGES;   // [2]: accumulator of panel parity b complete
+    uint64_t *xdone = accf + 2;        // one phase per panel: its columns solved and stored
+    uint32_t *tmem_slot = (uint32_t *)(xdone + 1);
+
+    const int m0 = blockIdx.x * BM;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    unsigned long long *flags = POTRF ? g_panel_flags[launch_id % kFlagSlots] : nullptr;
+    const unsigned long long tag = launch_id << 8;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < STAGES; s++) {
+            mbar_init(&full[s], NP / 32);
+            mbar_init(&empty[s], 1);
+        }
+        mbar_init(&accf[0], 1);
+        mbar_init(&accf[1], 1);
+        mbar_init(xdone, 4);
+        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    if (warp == 0) {
+        asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(tmem_slot)),
+                     "r"((uint32_t)(2 * P)));
+        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
+    }
+    tc_fence_before();
+    __syncthreads();
+    tc_fence_after();
+    const uint32_t tmem = *tmem_slot;
+    // panels this CTA takes part in: POTRF stops at the panel holding its rows' diagonal
+    int npanels = (n + P - 1) / P;
+    if (POTRF) npanels = min(npanels, (int)blockIdx.x + 1);
+
+    if (warp < 4) {
+        // =================================================== producers
+        const int t = threadIdx.x;
+        constexpr int APER = G::APER, BPER = G::BPER;
+        const float4 z4 = make_float4(0.f, 0.f, 0.f, 0.f);
+        int gkb = 0;
+        for (int J = 0; J < npanels; J++) {
+            const int c0 = J * P, nk = c0 / BK;
+            if (nk == 0) continue;
+            if (POTRF && J != (int)blockIdx.x) {
+                // panel J's L rows (CTA J's) are final once it completed panels < J
+                if (t == 0) wait_flag(&flags[J], tag | (unsigned long long)J);
+                asm volatile("bar.sync 1, 128;" ::: "memory");
+            }
+            // first k-block holding panel J-1's columns (overlap = 0: the whole panel waits)
+            const int kb_new = overlap ? nk - P / BK : 0;
+            constexpr uint32_t idesc = make_idesc(BM, P, false, false);
+            const uint32_t dt = tmem + (uint32_t)((J & 1) * P);
+            int kbp = 0;   // k-block of this panel being produced
+            bool waited = false;
+            auto ensure = [&](int kb) {
+                if (kb >= kb_new && !waited) {
+                    mbar_wait(xdone, (J - 1) & 1);   // panel J-1 solved and stored
+                    waited = true;
+                }
+            };
+            auto load = [&](float4 (&ra)[APER], float4 (&rb)[BPER], int kb) {
+                ensure(kb);
+                const int k0 = kb * BK;
+#pragma unroll
+                for (int p = 0; p < APER; p++) {
+                    const int f = t + p * NP, row = f >> 3, c = f & 7;
+                    ra[p] = (m0 + row < rows) ? ld_f4_cg(X + (int64_t)(m0 + row) * ldx + k0 + 4 * c) : z4;
+                }
+#pragma unroll
+                for (int p = 0; p < BPER; p++) {
+                    const int f = t + p * NP, row = f >> 3, c = f & 7;
+                    const float *src = L + (int64_t)(c0 + row) * ldl + k0 + 4 * c;
+                    rb[p] = (c0 + row < n) ? (POTRF ? ld_f4_cg(src) : __ldg(reinterpret_cast<const float4 *>(src))) : z4;
+                }
+            };
+            auto produce = [&](float4 (&ra)[APER], float4 (&rb)[BPER]) {
+                const int s = gkb % STAGES;
+                if (gkb >= STAGES) mbar_wait(&empty[s], ((gkb / STAGES) - 1) & 1);
+                uint8_t *st = smem + s * G::STAGE;
+                uint8_t *a_big = st, *a_small = st + G::A_BYTES;
+                uint8_t *b_big = st + 2 * G::A_BYTES, *b_small = b_big + G::B_BYTES;
+#pragma unroll
+                for (int p = 0; p < APER; p++) {
+                    const int f = t + p * NP, row = f >> 3, c = f & 7;
+                    store_split(a_big, a_small, kmaj_off(row, c), ra[p]);
+                }
+#pragma unroll
+                for (int p = 0; p < BPER; p++) {
+                    const int f = t + p * NP, row = f >> 3, c = f & 7;
+                    store_split(b_big, b_small, kmaj_off(row, c), rb[p]);
+                }
+                fence_proxy_async();
+                __syncwarp();
+                if (lane == 0) mbar_arrive(&full[s]);   // one release-arrive per producer warp
+                if (warp == 0) {
+                    // MMA issue: all four producer warps have filled stage s
+                    mbar_wait(&full[s], (gkb / STAGES) & 1);
+                    tc_fence_after();
+                    if (lane == 0) {
+                        const uint32_t ab = smem_u32(st), as = ab + G::A_BYTES;
+                        const uint32_t bb = ab + 2 * G::A_BYTES, bs = bb + G::B_BYTES;
+#pragma unroll
+                        for (int kk = 0; kk < BK / 8; kk++) {
+                            const uint32_t o = kk * 32;
+                            const uint64_t dAb = make_desc(ab + o, 16, 1024), dAs = make_desc(as + o, 16, 1024);
+                            const uint64_t dBb = make_desc(bb + o, 16, 1024), dBs = make_desc(bs + o, 16, 1024);
+                            const uint32_t first = (kbp == 0 && kk == 0) ? 0u : 1u;
+                            mma_tf32(dt, dAb, dBb, idesc, first);
+                            mma_tf32(dt, dAb, dBs, idesc, 1u);
+                            mma_tf32(dt, dAs, dBb, idesc, 1u);
+                        }
+                        mma_commit(&empty[s]);
+                        if (kbp == nk - 1) mma_commit(&accf[J & 1]);
+                    }
+                    __syncwarp();
+                }
+                kbp++;
+                gkb++;
+            };
+            float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
+            load(ra0, rb0, 0);
+            if (nk > 1) load(ra1, rb1, 1);
+            for (int kb = 0; kb < nk; kb += 2) {
+                produce(ra0, rb0);
+                if (kb + 2 < nk) load(ra0, rb0, kb + 2);
+                if (kb + 1 < nk) {
+                    produce(ra1, rb1);
+                    if (kb + 3 < nk) load(ra1, rb1, kb + 3);
+                }
+            }
+        }
+    } else {
+        // =================================================== epilogue (warps 4-7)
+        const int e = threadIdx.x - 128, row = m0 + e;
+        const uint32_t tl = tmem + ((uint32_t)((warp & 3) * 32) << 16);
+        const bool rowok = row < rows;
+        float *xrow = X + (int64_t)(rowok ? row : 0) * ldx;
+        uint32_t accn = 0;   // bit b: parity of the next accf[b] phase
+        for (int J = 0; J < npanels; J++) {
+            const int c0 = J * P, nk = c0 / BK, ncols = min(P, n - c0), nsb = ncols / PSB;
+            const uint32_t acc = tl + (uint32_t)((J & 1) * P);
+            const bool factor = POTRF && J == (int)blockIdx.x;
+            bar_epi();   // Lt / colbuf of the previous panel no longer read
+            if (!factor) {
+                if (POTRF) {
+                    if (e == 0) wait_flag(&flags[J], tag | (unsigned long long)(J + 1));
+                    bar_epi();
+                }
+                // stage L_JJ^T: rows q of L_JJ, coalesced in c = e; batched loads
+#pragma unroll 1
+                for (int q0 = 0; q0 < ncols; q0 += 32) {
+                    float tmp[32];
+#pragma unroll
+                    for (int q = 0; q < 32; q++) {
+                        const float *src = L + (int64_t)(c0 + q0 + q) * ldl + c0 + e;
+                        tmp[q] = (e <= q0 + q && e < ncols) ? (POTRF ? ld_f_cg(src) : __ldg(src)) : 0.f;
+                    }
+#pragma unroll
+                    for (int q = 0; q < 32; q++) Lt[e * LD + q0 + q] = tmp[q];
+                }
+                if (e < ncols) Lr[e] = rcp_approx(Lt[e * LD + e]);   // this thread's own store
+                bar_epi();
+            }
+            // b values of sub-block 0 (the tile's current values of the panel columns)
+            float4 bq[4], bn[4];
+#pragma unroll
+            for (int q = 0; q < 4; q++) bq[q] = rowok ? ld_f4_cg(xrow + c0 + 4 * q) : make_float4(0.f, 0.f, 0.f, 0.f);
+            if (nk > 0) {
+                mbar_wait(&accf[J & 1], (accn >> (J & 1)) & 1u);
+                accn ^= 1u << (J & 1);
+                tc_fence_after();
+            } else {
+                float z[16];
+#pragma unroll
+                for (int i = 0; i < 16; i++) z[i] = 0.f;
+#pragma unroll 1
+                for (int sb = 0; sb < nsb; sb++) tmem_st16(acc + sb * PSB, z);
+            }
+#pragma unroll 1
+            for (int sb = 0; sb < nsb; sb++) {
+                if (sb + 1 < nsb) {
+#pragma unroll
+                    for (int q = 0; q < 4; q++)
+                        bn[q] = rowok ? ld_f4_cg(xrow + c0 + (sb + 1) * PSB + 4 * q) : make_float4(0.f, 0.f, 0.f, 0.f);
+                }
+                float x[PSB];
+                tmem_ld16(acc + sb * PSB, x);
+#pragma unroll
+                for (int q = 0; q < 4; q++) {
+                    x[4 * q + 0] = bq[q].x - x[4 * q + 0];
+                    x[4 * q + 1] = bq[q].y - x[4 * q + 1];
+                    x[4 * q + 2] = bq[q].z - x[4 * q + 2];
+                    x[4 * q + 3] = bq[q].w - x[4 * q + 3];
+                }
+                if (factor) {
+#pragma unroll
+                    for (int c = 0; c < PSB; c++) {
+                        const int pr = sb * PSB + c;   // pivot row / column within the block
+                        if (e == pr) {
+                            const float piv = x[c];
+                            if (!(piv > 0.f) && info) atomicCAS(info, 0, k_base + c0 + pr + 1);
+                            x[c] = sqrtf(piv);
+                            pivot = x[c];
+                        }
+                        bar_epi();
+                        const float l = pivot;
+                        if (e > pr) {
+                            x[c] = div_nr(x[c], l, rcp_approx(l));
+                            colbuf[e] = x[c];
+                        }
+                        bar_epi();
+                        if (e > pr) {
+#pragma unroll
+                            for (int j = c + 1; j < PSB; j++) x[j] = fmaf(-x[c], colbuf[sb * PSB + j], x[j]);
+                        }
+                    }
+                    // publish this row's L_JJ values (transposed) for the cross updates
+#pragma unroll
+                    for (int c = 0; c < PSB; c++) Lt[(sb * PSB + c) * LD + e] = x[c];
+                    bar_epi();
+                } else {
+#pragma unroll
+                    for (int c = 0; c < PSB; c++) {
+                        const int cc = sb * PSB + c;
+                        x[c] = div_nr(x[c], Lt[cc * LD + cc], Lr[cc]);
+#pragma unroll
+                        for (int j = c + 1; j < PSB; j++) x[j] = fmaf(-x[c], Lt[cc * LD + sb * PSB + j], x[j]);
+                    }
+                }
+                // store the solved row segment (diagonal block: lower part only)
+                if (rowok) {
+                    float *dst = xrow + c0 + sb * PSB;
+                    if (factor) {
+#pragma unroll
+                        for (int c = 0; c < PSB; c++)
+                            if (sb * PSB + c <= e) dst[c] = x[c];
+                    } else {
+#pragma unroll
+                        for (int q = 0; q < PSB / 4; q++)
+                            *reinterpret_cast<float4 *>(dst + 4 * q) =
+                                make_float4(x[4 * q], x[4 * q + 1], x[4 * q + 2], x[4 * q + 3]);
+                    }
+                }
+                // acc[tb] += x L[tb, sb]^T for the later sub-blocks; TMEM loads one
+                // sub-block ahead, stores unwaited until the next sub-block reads TMEM
+                if (sb + 1 < nsb) {
+                    float a[PSB], an[PSB];
+                    tmem_ld16_issue(acc + (sb + 1) * PSB, a);
+                    tmem_wait_ld(a);
+#pragma unroll 1
+                    for (int tb = sb + 1; tb < nsb; tb++) {
+                        if (tb + 1 < nsb) tmem_ld16_issue(acc + (tb + 1) * PSB, an);
+#pragma unroll
+                        for (int c = 0; c < PSB; c++) {
+                            const float *lc = Lt + (sb * PSB + c) * LD + tb * PSB;
+#pragma unroll
+                            for (int q = 0; q < PSB / 4; q++) {
+                                const float4 l4 = *reinterpret_cast<const float4 *>(lc + 4 * q);
+                                a[4 * q + 0] = fmaf(x[c], l4.x, a[4 * q + 0]);
+                                a[4 * q + 1] = fmaf(x[c], l4.y, a[4 * q + 1]);
+                                a[4 * q + 2] = fmaf(x[c], l4.z, a[4 * q + 2]);
+                                a[4 * q + 3] = fmaf(x[c], l4.w, a[4 * q + 3]);
+                            }
+                        }
+                        tmem_st16_issue(acc + tb * PSB, a);
+                        if (tb + 1 < nsb) {
+                            tmem_wait_ld(an);
+#pragma unroll
+                            for (int i = 0; i < PSB; i++) a[i] = an[i];
+                        }
+                    }
+                    tmem_wait_st();
+                }
+#pragma unroll
+                for (int q = 0; q < 4; q++) bq[q] = bn[q];
+            }
+            // panel J of these rows: visible at L2 (own producers, other CTAs), TMEM reads done
+            __threadfence();
+            tc_fence_before();
+            __syncwarp();
+            if (lane == 0) mbar_arrive(xdone);
+            if (POTRF) {
+                bar_epi();
+                if (e == 0) st_release(&flags[blockIdx.x], tag | (unsigned long long)(J + 1));
+            }
+        }
+    }
+
+    tc_fence_before();
+    __syncthreads();
+    tc_fence_after();
+    if (warp == 0) {
+        asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)(2 * P)));
+    }
+    ctx_end(ctx);
+}
+
+// MMA of panel J+1 overlapped with the solve of panel J (default); VS_PANEL_OVERLAP=0
+// serialises them (measurement switch)
+inline int panel_overlap()
+{
+    static const int v = [] {
+        const char *e = getenv("VS_PANEL_OVERLAP");
+        return e ? atoi(e) : 1;
+    }();
+    return v;
+}
+
+template <bool POTRF>
+inline void panel_attr()
+{
+    static bool attr[64] = {};
+    int dev = 0;
+    cudaGetDevice(&dev);
+    if (!attr[dev & 63]) {
+        cudaFuncSetAttribute(tc_panel_kernel<POTRF>, cudaFuncAttributeMaxDynamicSharedMemorySize, PanelCfg::SMEM);
+        attr[dev & 63] = true;
+    }
+}
+
+// X <- X L^{-T}: rows x n (n % 64 == 0), one launch.
+inline int tc_trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, cudaStream_t s,
+                   const TaskCtx &ctx = TaskCtx())
+{
+    if (rows <= 0 || n <= 0) return 0;
+    if (n % 64) return -1;
+    panel_attr<false>();
+    count_launch();
+    tc_panel_kernel<false><<<(rows + BM - 1) / BM, PTHREADS, PanelCfg::SMEM, s>>>(rows, n, L, ldl, X, ldx, 0, nullptr,
+                                                                                  0ull, panel_overlap(), ctx);
+    return 0;
+}
+
+// A = L L^T in place: n x n (n % 64 == 0, n <= 4096), one launch.
+inline int tc_potrf(int n, float *A, int lda, int k_base, int *info, cudaStream_t s, const TaskCtx &ctx = TaskCtx())
+{
+    if (n <= 0) return 0;
+    if (n % 64 || (n + BM - 1) / BM > kFlagCtas) return -1;
+    static std::atomic<unsigned long long> next_id{1};
+    const unsigned long long id = next_id.fetch_add(1);
+    panel_attr<true>();
+    count_launch();
+    tc_panel_kernel<true><<<(n + BM - 1) / BM, PTHREADS, PanelCfg::SMEM, s>>>(n, n, A, lda, A, lda, k_base, info, id,
+                                                                             panel_overlap(), ctx);
+    return 0;
+}
+
+}  // namespace tc
+}  // namespace vsk
