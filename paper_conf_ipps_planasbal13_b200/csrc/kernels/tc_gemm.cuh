@@ -200,8 +200,7 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
     uint64_t *full = (uint64_t *)(smem + STAGES * G::STAGE);
     uint64_t *empty = full + STAGES;
     uint64_t *acc_full = empty + STAGES;
-    uint64_t *c_ready = acc_full + 1;
-    uint32_t *tmem_slot = (uint32_t *)(c_ready + 1);
+    uint32_t *tmem_slot = (uint32_t *)(acc_full + 1);
 
     const int m0 = blockIdx.y * BM, n0 = blockIdx.x * BN;
     if (LOWER && n0 >= m0 + BM) {
@@ -217,7 +216,6 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
             mbar_init(&empty[s], 1);
         }
         mbar_init(acc_full, 1);
-        mbar_init(c_ready, NPROD);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     }
     if (warp == NPROD / 32) {
@@ -295,16 +293,13 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
             __syncwarp();                            // the warp's stores + fences precede...
             if (lane == 0) mbar_arrive(&full[s]);    // ...one release-arrive per warp
         };
-        // two k-blocks of loads in flight (register double buffer, loop unrolled by 2)
-        float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
-        load(ra0, rb0, 0);
-        if (nk > 1) load(ra1, rb1, 1);
-        // preload the C tile into the TMEM accumulator (this warp: lane quarter eq, column
-        // half eh) while the first k-blocks are in flight; the MMAs then accumulate onto it
+        // C_in staging into TMEM columns [BN, 2BN) (this warp: lane quarter eq, column half
+        // eh), one 32-column chunk after each of the first k-blocks so that the MMAs start
+        // at once and the chunk loads hide behind the queued stages
         const int eq = warp & 3, eh = warp >> 2;
         const int erow = m0 + eq * 32 + lane;
-#pragma unroll 1
-        for (int c = 0; c < BN / 64; c++) {
+        constexpr int NCH = BN / 64;
+        auto stage_c = [&](int c) {
             const int col0 = eh * (BN / 2) + c * 32;
             float v[32];
             const float *crow = C + (int64_t)erow * ldc + n0 + col0;
@@ -314,18 +309,24 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
                 v[4 * j] = x.x; v[4 * j + 1] = x.y; v[4 * j + 2] = x.z; v[4 * j + 3] = x.w;
             }
             tmem_st32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(BN + col0), v);
-        }
-        asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
-        tc_fence_before();
-        mbar_arrive(c_ready);
+        };
+        // two k-blocks of loads in flight (register double buffer, loop unrolled by 2)
+        float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
+        load(ra0, rb0, 0);
+        if (nk > 1) load(ra1, rb1, 1);
+        int staged = 0;
         for (int kb = 0; kb < nk; kb += 2) {
             produce(ra0, rb0, kb);
             if (kb + 2 < nk) load(ra0, rb0, kb + 2);
+            if (staged < NCH) stage_c(staged++);
             if (kb + 1 < nk) {
                 produce(ra1, rb1, kb + 1);
                 if (kb + 3 < nk) load(ra1, rb1, kb + 3);
+                if (staged < NCH) stage_c(staged++);
             }
         }
+        while (staged < NCH) stage_c(staged++);
+        asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
 
         // ------------------------------------------------------------ epilogue
         mbar_wait(acc_full, 0);
