@@ -37,7 +37,7 @@ SEED_MM, SEED_CH = 3, 4
 # runtime configuration the bench times (env VS_SLOTS / VS_PRIORITY / VS_QDEPTH override):
 # lambda 3, 6 workers (streams) per GPU, NEXT-4 bottom-level priority with queue depth 2
 RT_DEFAULTS = dict(lam=3, slots=6, priority=2, qdepth=2)
-F32_VERSIONS_MASK = 0b111     # simt_f32 | tc_3xtf32 | f64in_f32io
+F32_VERSIONS_MASK = 0b100111  # simt_f32 | tc_3xtf32 | f64in_f32io | tc_3xf16 (gemm-type tasks)
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
 
@@ -131,18 +131,20 @@ class Workload:
         return T, [ids[t] for t in tiles]
 
     def reset(self):
-        """Restore this rank's inputs (C = 0, A_chol = pristine).  Device: async on torch's
-        stream + sync.  Host (e2e): memcpy, then every datum is declared modified so the
-        runtime re-transfers it (the e2e timed region includes those copies)."""
+        """Restore this rank's inputs (C = 0, A_chol = pristine) and declare EVERY datum
+        modified (vs_data_invalidate), as if a new batch of inputs had been written: no
+        replica, cached remote tile or derived operand form (tc_3xf16 split halves) of the
+        previous step is reused, so each step re-does all moves and conversions.  Device:
+        async on torch's stream + sync.  Host (e2e): memcpy; the runtime re-transfers every
+        tile (the e2e timed region includes those copies)."""
         if self.with_mm:
             self.C.zero_()
         if self.with_ch:
             self.S.copy_(self.S0)
-        if self.host:
-            for d in self.ids:
-                self.rt.vs_data_invalidate(d)
-        else:
+        if not self.host:
             self.torch.cuda.current_stream().synchronize()
+        for d in self.ids:
+            self.rt.vs_data_invalidate(d)
 
     def submit(self):
         vs, rt = self.vs, self.rt
@@ -242,14 +244,18 @@ def roofline(log, groups, ms, world):
     dom = max(per, key=lambda k: per[k]["flops"])
     d = per[dom]
     union = union_ns(d["iv"])
-    hw = 3.0 if dom[1] == "tc_3xtf32" else 1.0
+    f16_peak = pk.get("bf16_tflops_sustained", pk["bf16_tflops"])            # fp16 dense = bf16 dense rate
+    tc_peak = {"tc_3xtf32": (tf32_peak, "%s bf16_tflops_sustained x 0.5 (TF32/BF16 nominal ratio)" % pk_kind),
+               "tc_3xf16": (f16_peak, "%s bf16_tflops_sustained (fp16 = bf16 dense rate)" % pk_kind)}
+    hw = 3.0 if dom[1] in tc_peak else 1.0
     achieved = hw * d["flops"] / (union * 1e-9) / 1e12
-    if dom[1] == "tc_3xtf32":
-        peak, bound, src = tf32_peak, "tensor", "%s bf16_tflops_sustained x 0.5 (TF32/BF16 nominal ratio)" % pk_kind
+    if dom[1] in tc_peak:
+        (peak, src), bound = tc_peak[dom[1]], "tensor"
     else:
         peak, bound, src = 148 * 128 * 2 * pk["sm_max_mhz"] * 1e6 / 1e12, "alu", "148 SM x 128 FMA x 2 x sm_max_mhz"
-    tc_flops = sum(v["flops"] for k, v in per.items() if k[1] == "tc_3xtf32")
-    frac_step = 3.0 * tc_flops / (ms * 1e-3) / 1e12 / tf32_peak
+    # tensor-pipe busy fraction of the whole step: hardware MMA flops of every tensor-core
+    # task / (step time x that version's peak), summed over versions
+    frac_step = sum(3.0 * v["flops"] / tc_peak[k[1]][0] for k, v in per.items() if k[1] in tc_peak) / (ms * 1e-3) / 1e12
     roof = {"bound": bound, "kernel": "%s/%s b=%d" % dom, "achieved": round(achieved, 2), "peak": round(peak, 1),
             "unit": "TFLOP/s", "frac": round(achieved / peak, 4), "traffic": None, "peak_source": src,
             "how": "hardware MMA flops (3x algorithmic) of all launches of this kernel class in the timed steps / "
@@ -479,7 +485,7 @@ def main():
             "higher_is_better": True, "scaling": "strong" if world > 1 else "weak", "vs_baseline": None, "dtype": "f32",
             "data": "synthetic (counter-based generator; U(-1,1) matmul operands, SPD A = S + 2.5 sqrt(N) I)",
             "config": {"workload": ("cfg3+cfg4: tiled matmul N=%d b=%d + tiled Cholesky N=%d b=%d, fp32, versions "
-                                    "simt_f32/tc_3xtf32/f64in_f32io, lambda=%d, %d slots/GPU" % (
+                                    "simt_f32/tc_3xtf32/f64in_f32io/tc_3xf16, lambda=%d, %d slots/GPU" % (
                                         mm_n, mm_b, ch_n, ch_b, args.lam, args.slots)) if with_mm and with_ch else
                        args.only,
                        "matmul_N": mm_n if with_mm else None, "cholesky_N": ch_n if with_ch else None,
@@ -497,6 +503,7 @@ def main():
             "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "mode": "runahead"},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
+            "operand_forms_per_step": int((st1.forms_built - st0.forms_built) / args.steps),
             "device_tx_bytes_per_step": int((st1.device_tx_bytes - st0.device_tx_bytes) / args.steps),
             "host_us_per_task": {"decide": round((st1.host_ns_decide - st0.host_ns_decide) / 1e3 / max(1, len(log)), 3),
                                  "issue": round((st1.host_ns_issue - st0.host_ns_issue) / 1e3 / max(1, len(log)), 3)},

@@ -96,7 +96,11 @@ enum {
     VS_V_F64IN_F32IO = 2, /* fp32 in/out, fp64 arithmetic (DMMA), one rounding on store */
     VS_V_DFMA_F64 = 3,    /* fp64 tiles, SIMT DFMA */
     VS_V_DMMA_F64 = 4,    /* fp64 tiles, mma.sync f64 tensor cores */
-    VS_NUM_BUILTIN_VERSIONS = 5
+    VS_V_TC_3XF16 = 5,    /* fp32 tiles, tcgen05 kind::f16 on row-scaled fp16 big/small halves of the
+                             operands (reading R30); MATMUL, GEMM_NT and SYRK only.  Its in-operands
+                             are read through a per-GPU cached "split form" that the runtime builds
+                             (one conversion kernel per datum version, like a tile move) */
+    VS_NUM_BUILTIN_VERSIONS = 6
 };
 
 typedef struct {
@@ -174,7 +178,8 @@ int vs_version_add(vs_rt rt, vs_type_id type, const char *name, uint32_t gpu_mas
                    vs_launch_fn fn, void *user, vs_version_id *out);
 
 /* Register the five built-in tile task types for dtype (VS_F32: versions SIMT_F32,
- * TC_3XTF32, F64IN_F32IO; VS_F64: DFMA_F64, DMMA_F64), keeping the versions whose
+ * TC_3XTF32, F64IN_F32IO, TC_3XF16 (MATMUL/GEMM_NT/SYRK only); VS_F64: DFMA_F64,
+ * DMMA_F64), keeping the versions whose
  * bit is set in version_mask (bit = VS_V_*).  out_types[VS_T_*] receives the type ids;
  * version index order inside each type follows increasing VS_V_* id.  Runnable on
  * every gpu.  Errors: VS_E_INVAL if no version of dtype is selected. */
@@ -188,7 +193,8 @@ int vs_register_builtins(vs_rt rt, int dtype, uint32_t version_mask,
 int vs_data_register(vs_rt rt, void *ptr, int device, int64_t bytes, vs_data_id *out);
 
 /* The caller modified datum d at its home outside any task (after a wait): every other
- * copy (device replica, cached remote copy) is stale and will be re-fetched on next use.
+ * copy (device replica, cached remote copy, derived operand form) is stale and will be
+ * re-fetched / rebuilt on next use.  Callers MUST call it after such a modification.
  * VS_E_STATE if a task writing d is still in flight. */
 int vs_data_invalidate(vs_rt rt, vs_data_id d);
 
@@ -219,6 +225,7 @@ typedef struct {
     int64_t kernel_launches;  /* process-wide count of libvsched kernel launches */
     int64_t tracker;          /* dependence tracker in use: 1 = device completion words
                                  (stream memory operations), 0 = CUDA events */
+    int64_t forms_built;      /* derived operand forms built (VS_V_TC_3XF16 split halves) */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 
@@ -284,6 +291,19 @@ int vs_app_cholesky(vs_rt rt, const vs_type_id types[VS_NUM_BUILTIN_TYPES], int 
  * (may be NULL for other types).  Returns VS_E_INVAL for an unknown (type, version)
  * or an unsupported b (b must be a multiple of 32, 32 <= b <= 4096). */
 int vs_tile_run(int type, int version, int b, void *const *ptrs, int *dinfo, void *stream);
+
+/* Derived operand forms (reading R30).  vs_operand_form returns the form (0 = the tile
+ * itself, 1 = row split form, 2 = column split form, i.e. the row split form of the
+ * transposed tile) in which `version` reads parameter `param` of built-in `type`;
+ * vs_form_bytes the size of a form of a b x b fp32 tile (0 for form 0).
+ * vs_form_make enqueues the conversion of the b x b fp32 tile `src` into `dst`
+ * (vs_form_bytes bytes, device memory, 16-byte aligned) on `stream`.
+ * vs_tile_run_prepared is vs_tile_run with ptrs[param] already in its form (no
+ * conversion): the kernel the runtime launches for a task.  VS_E_INVAL on bad arguments. */
+int vs_operand_form(int type, int version, int param);
+int64_t vs_form_bytes(int form, int b);
+int vs_form_make(int form, int b, const void *src, void *dst, void *stream);
+int vs_tile_run_prepared(int type, int version, int b, void *const *ptrs, int *dinfo, void *stream);
 
 /* ---------------------------------------------------------- input generator */
 /* Device counter-based generator, bit-identical to vsgen.uniform_idx:

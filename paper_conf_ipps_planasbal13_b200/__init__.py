@@ -27,9 +27,9 @@ VS_POLICY_VERSIONING, VS_POLICY_FIXED = 0, 1
 VS_F32, VS_F64 = 0, 1
 VS_T_MATMUL, VS_T_POTRF, VS_T_TRSM, VS_T_SYRK, VS_T_GEMM_NT = range(5)
 VS_NUM_BUILTIN_TYPES = 5
-VS_V_SIMT_F32, VS_V_TC_3XTF32, VS_V_F64IN_F32IO, VS_V_DFMA_F64, VS_V_DMMA_F64 = range(5)
+VS_V_SIMT_F32, VS_V_TC_3XTF32, VS_V_F64IN_F32IO, VS_V_DFMA_F64, VS_V_DMMA_F64, VS_V_TC_3XF16 = range(6)
 VS_MAX_VERSIONS = 8
-VERSION_NAMES = ["simt_f32", "tc_3xtf32", "f64in_f32io", "dfma_f64", "dmma_f64"]
+VERSION_NAMES = ["simt_f32", "tc_3xtf32", "f64in_f32io", "dfma_f64", "dmma_f64", "tc_3xf16"]
 TYPE_NAMES = ["MATMUL", "POTRF", "TRSM", "SYRK", "GEMM_NT"]
 
 ERRORS = {0: "VS_OK", -1: "VS_E_INVAL", -2: "VS_E_NOMEM", -3: "VS_E_CUDA", -4: "VS_E_NOT_SPD",
@@ -48,7 +48,7 @@ class vs_stats_t(Structure):
     _fields_ = [(n, c_int64) for n in (
         "tasks_submitted", "tasks_completed", "decisions", "input_tx_bytes", "output_tx_bytes", "device_tx_bytes",
         "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns",
-        "kernel_launches", "tracker")]
+        "kernel_launches", "tracker", "forms_built")]
 
 
 class vs_group_stat_t(Structure):
@@ -122,6 +122,10 @@ def lib():
         "vs_ipc_open": (c_int, [ctypes.c_char * 64, c_uint64, POINTER(c_void_p)]),
         "vs_ipc_close": (c_int, [c_void_p]),
         "vs_data_invalidate": (c_int, [rt, c_int64]),
+        "vs_operand_form": (c_int, [c_int, c_int, c_int]),
+        "vs_form_bytes": (c_int64, [c_int, c_int]),
+        "vs_form_make": (c_int, [c_int, c_int, c_void_p, c_void_p, c_void_p]),
+        "vs_tile_run_prepared": (c_int, [c_int, c_int, c_int, POINTER(c_void_p), c_void_p, c_void_p]),
     }
     for name, (res, args) in sig.items():
         f = getattr(L, name)
@@ -137,7 +141,8 @@ EXPORTED = ["vs_config_default", "vs_create", "vs_destroy", "vs_last_error", "vs
             "vs_decision_log", "vs_decision_log_hash", "vs_decision_log_clear", "vs_table_dump", "vs_table_load",
             "vs_replay_set", "vs_app_matmul", "vs_app_cholesky", "vs_tile_run", "vs_gen_uniform", "vs_gen_spd",
             "vs_build_info", "vs_gen_tile", "vs_dist_init", "vs_data_set_owner", "vs_ipc_export", "vs_ipc_open",
-            "vs_ipc_close", "vs_data_invalidate"]
+            "vs_ipc_close", "vs_data_invalidate", "vs_operand_form", "vs_form_bytes", "vs_form_make",
+            "vs_tile_run_prepared"]
 
 
 def _ids(seq, ctype=c_int64):
@@ -160,6 +165,28 @@ def vs_tile_run(ttype, version, b, ptrs, dinfo=0, stream=0):
     r = lib().vs_tile_run(ttype, version, b, arr, c_void_p(dinfo or None), c_void_p(stream or None))
     if r:
         raise VSError(r, "vs_tile_run(type=%d, version=%d, b=%d)" % (ttype, version, b))
+
+
+def vs_operand_form(ttype, version, param):
+    return lib().vs_operand_form(ttype, version, param)
+
+
+def vs_form_bytes(form, b):
+    return lib().vs_form_bytes(form, b)
+
+
+def vs_form_make(form, b, src_ptr, dst_ptr, stream=0):
+    r = lib().vs_form_make(form, b, c_void_p(src_ptr), c_void_p(dst_ptr), c_void_p(stream or None))
+    if r:
+        raise VSError(r, "vs_form_make(form=%d, b=%d)" % (form, b))
+
+
+def vs_tile_run_prepared(ttype, version, b, ptrs, dinfo=0, stream=0):
+    """vs_tile_run with the operands already in the version's forms (vs_operand_form)."""
+    arr = (c_void_p * len(ptrs))(*ptrs)
+    r = lib().vs_tile_run_prepared(ttype, version, b, arr, c_void_p(dinfo or None), c_void_p(stream or None))
+    if r:
+        raise VSError(r, "vs_tile_run_prepared(type=%d, version=%d, b=%d)" % (ttype, version, b))
 
 
 def vs_gen_uniform(seed, rows, cols, dtype, tile_b, dev_ptr, stream=0):

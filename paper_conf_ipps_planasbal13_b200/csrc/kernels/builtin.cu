@@ -9,6 +9,7 @@
 //   f64in_f32io    fp32     dmma_gemm<float>  (DMMA on upcast operands)            blocked
 //   dfma_f64       fp64     simt_gemm<double,double> (DFMA)                        blocked
 //   dmma_f64       fp64     dmma_gemm<double>  (mma.sync f64)                      blocked
+//   tc_3xf16       fp32     tcf_gemm (tcgen05 kind::f16 on split forms, tc_f16.cuh) (gemm types only)
 //
 // potrf of tc_3xtf32 is the single-launch left-looking tc_panel kernel (tc_panel.cuh).
 // potrf of the other versions is recursive: potrf(A11); A21 <- A21 L11^{-T} (trsm);
@@ -22,6 +23,7 @@
 #include "simt_chol.cuh"
 #include "simt_gemm.cuh"
 #include "tc_gemm.cuh"
+#include "tc_f16.cuh"
 #include "tc_panel.cuh"
 
 #include "vsched.h"
@@ -140,15 +142,49 @@ int run_family(int type, int b, void *const *p, int *info, cudaStream_t s, const
 
 }  // namespace
 
-int builtin_elem_bytes(int version) { return version >= VS_V_DFMA_F64 ? 8 : 4; }
+int builtin_elem_bytes(int version) { return (version == VS_V_DFMA_F64 || version == VS_V_DMMA_F64) ? 8 : 4; }
 
 bool builtin_supported(int type, int version, int b)
 {
     if (type < 0 || type >= VS_NUM_BUILTIN_TYPES) return false;
     if (version < 0 || version >= VS_NUM_BUILTIN_VERSIONS) return false;
+    if (version == VS_V_TC_3XF16 && (type == VS_T_POTRF || type == VS_T_TRSM)) return false;
     if (b && (b % 64 != 0 || b < 64 || b > 4096)) return false;
     return true;
 }
+
+int builtin_operand_form(int type, int version, int param)
+{
+    if (version != VS_V_TC_3XF16) return FORM_RAW;
+    switch (type) {
+    case VS_T_MATMUL: return param == 0 ? FORM_SPLIT_ROWS : param == 1 ? FORM_SPLIT_COLS : FORM_RAW;
+    case VS_T_GEMM_NT: return param <= 1 ? FORM_SPLIT_ROWS : FORM_RAW;
+    case VS_T_SYRK: return param == 0 ? FORM_SPLIT_ROWS : FORM_RAW;
+    }
+    return FORM_RAW;
+}
+
+size_t form_bytes(int form, int b) { return form == FORM_RAW ? 0 : tcf::split_bytes(b, b); }
+
+int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
+{
+    if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
+    if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
+    return -1;
+}
+
+namespace {
+// tc_3xf16: p[] holds the split forms of the in-operands (builtin_operand_form)
+int run_f16(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
+{
+    switch (type) {
+    case VS_T_MATMUL: return tcf::tcf_gemm<false, false>(b, b, b, p[0], p[1], (float *)p[2], b, s, ctx);
+    case VS_T_GEMM_NT: return tcf::tcf_gemm<true, false>(b, b, b, p[0], p[1], (float *)p[2], b, s, ctx);
+    case VS_T_SYRK: return tcf::tcf_gemm<true, true>(b, b, b, p[0], p[0], (float *)p[1], b, s, ctx);
+    }
+    return -1;
+}
+}  // namespace
 
 int launch_builtin(int type, int version, int b, void *const *p, int *info, cudaStream_t s, const TaskCtx &ctx)
 {
@@ -159,6 +195,7 @@ int launch_builtin(int type, int version, int b, void *const *p, int *info, cuda
     case VS_V_F64IN_F32IO: return run_family<float, DmmaEngine<float>>(type, b, p, info, s, ctx);
     case VS_V_DFMA_F64: return run_family<double, SimtEngine<double, double>>(type, b, p, info, s, ctx);
     case VS_V_DMMA_F64: return run_family<double, DmmaEngine<double>>(type, b, p, info, s, ctx);
+    case VS_V_TC_3XF16: return run_f16(type, b, p, s, ctx);
     }
     return -1;
 }

@@ -32,6 +32,14 @@ bool builtin_supported(int type, int version, int b);
 // Element size in bytes for a version (4 for f32-io versions, 8 for f64).
 int builtin_elem_bytes(int version);
 
+// Operand forms: a version may read an in-parameter through a derived copy of the tile
+// that the runtime builds and caches per (datum version, GPU), like a replica (a8).
+enum { FORM_RAW = 0, FORM_SPLIT_ROWS = 1, FORM_SPLIT_COLS = 2, NUM_FORMS = 3 };
+int builtin_operand_form(int type, int version, int param);
+size_t form_bytes(int form, int b);
+// Build the form of the b x b fp32 tile src into dst (form_bytes) on stream s.
+int make_form(int form, int b, const void *src, void *dst, cudaStream_t s);
+
 int gen_uniform(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b, void *out,
                 cudaStream_t s);
 int gen_spd(uint64_t seed, int64_t n, int dtype, int tile_b, void *out, cudaStream_t s);

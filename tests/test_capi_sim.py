@@ -15,7 +15,7 @@ ALL = 0xFFFF
 def test_library_exports_every_header_symbol():
     L = vs.lib()
     hdr = open(os.path.join(ROOT, "include", "vsched.h")).read()
-    names = set(re.findall(r"^(?:int|void|uint64_t|const char \*)\s*(vs_[a-z_0-9]+)\(", hdr, re.M))
+    names = set(re.findall(r"^(?:int|void|uint64_t|int64_t|const char \*)\s*(vs_[a-z_0-9]+)\(", hdr, re.M))
     assert len(names) >= 25
     for n in sorted(names):
         assert hasattr(L, n), n

@@ -171,3 +171,62 @@ def test_replay_mode_bit_exact_outputs(gpu):
         rt.close()
     assert hashes[0] == hashes[1]
     assert np.array_equal(outs[0].view(np.uint32), outs[1].view(np.uint32))
+
+
+F16_MASK = F32_MASK | (1 << vs.VS_V_TC_3XF16)
+
+
+def test_tc_3xf16_versioning_matmul_and_cholesky(gpu):
+    # tc_3xf16 competes with the other fp32 versions for MATMUL / GEMM_NT / SYRK (POTRF and
+    # TRSM keep three versions); every version's output is within the fp32-class gate (R22).
+    rt = vs.Runtime(lam=2)
+    C0 = vsgen.uniform(2002, 1024, 1024)
+    A, B, C0, C = _matmul(rt, 1024, 256, mask=F16_MASK, C0=C0)
+    assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-5
+    g = rt.vs_group_stats()[0]
+    assert g["versions"] == ["simt_f32", "tc_3xtf32", "f64in_f32io", "tc_3xf16"]
+    assert g["n"][3] >= 2
+    rt.close()
+    rt = vs.Runtime(lam=2)
+    A, L = _cholesky(rt, 2048, 256, mask=F16_MASK)
+    Lref, info = oracle.cholesky(A)
+    lo, slo = np.tril_indices(2048), np.tril_indices(2048, -1)
+    assert info == 0 and oracle.relF(L[lo], Lref[lo]) <= 1e-5 and oracle.relF(L[slo], Lref[slo]) <= 1e-5
+    gs = {gr["type_name"]: gr for gr in rt.vs_group_stats()}
+    assert len(gs["POTRF.f32"]["versions"]) == 3 and len(gs["GEMM_NT.f32"]["versions"]) == 4
+    assert rt.vs_stats().forms_built > 0
+    rt.close()
+
+
+def test_tc_3xf16_forms_follow_writes_and_invalidation(gpu):
+    # The split forms are cached per datum version: a task write (C of step 1 becomes the A
+    # operand of step 2) and vs_data_invalidate after an outside write must both rebuild them.
+    torch = _torch()
+    N, b = 512, 128
+    nt = N // b
+    rt = vs.Runtime(vs.vs_config_default(lam=1, policy=vs.VS_POLICY_FIXED, fixed_version=3))
+    types = rt.vs_register_builtins(vs.VS_F32, F16_MASK)
+    A, B = vsgen.uniform(31, N, N), vsgen.uniform(32, N, N)
+    tA, tB, tC, tD = (_tiles_dev(x, b) for x in (A, B, np.zeros((N, N), np.float32), np.zeros((N, N), np.float32)))
+    ia, ib, ic, idd = (_register_tiles(rt, t) for t in (tA, tB, tC, tD))
+    mm = types[vs.VS_T_MATMUL]
+    rt.vs_app_matmul(mm, nt, nt, nt, ia, ib, ic)       # C = A B
+    rt.vs_app_matmul(mm, nt, nt, nt, ic, ib, idd)      # D = C B (reads C's new content)
+    rt.vs_wait_all()
+    C = A.astype(np.float64) @ B
+    D = C @ B
+    assert oracle.relF(vsgen.from_tiles(tD.cpu().numpy()), D) <= 1e-5
+    n1 = rt.vs_stats().forms_built
+    assert n1 == 3 * nt * nt                             # A, B, C once each
+    # outside write of A + invalidate -> rebuilt; B unchanged -> reused
+    A2 = vsgen.uniform(33, N, N)
+    tA.copy_(_tiles_dev(A2, b))
+    tC.zero_()
+    torch.cuda.synchronize()
+    for d in ia + ic:
+        rt.vs_data_invalidate(d)
+    rt.vs_app_matmul(mm, nt, nt, nt, ia, ib, ic)
+    rt.vs_wait_all()
+    assert oracle.relF(vsgen.from_tiles(tC.cpu().numpy()), A2.astype(np.float64) @ B) <= 1e-5
+    assert rt.vs_stats().forms_built == n1 + nt * nt
+    rt.close()

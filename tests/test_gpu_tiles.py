@@ -12,6 +12,7 @@ pytestmark = pytest.mark.gpu
 
 F32_VERSIONS = [vs.VS_V_SIMT_F32, vs.VS_V_TC_3XTF32, vs.VS_V_F64IN_F32IO]
 F64_VERSIONS = [vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64]
+GEMM_VERSIONS = F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS   # tc_3xf16: gemm-type tasks only
 SIZES = [64, 128, 192, 320, 512]
 
 
@@ -65,7 +66,7 @@ def test_device_generator_bit_identical(gpu):
 
 
 # ------------------------------------------------------------------ matmul / gemm / syrk
-@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("version", GEMM_VERSIONS)
 @pytest.mark.parametrize("b", SIZES)
 def test_matmul_tile(gpu, version, b):
     dt = _dt(version)
@@ -75,7 +76,7 @@ def test_matmul_tile(gpu, version, b):
     assert oracle.relF(C, ref) <= _gate(version)
 
 
-@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("version", GEMM_VERSIONS)
 @pytest.mark.parametrize("b", SIZES)
 def test_gemm_nt_and_syrk_tiles(gpu, version, b):
     dt = _dt(version)
@@ -101,7 +102,7 @@ def test_simt_f32_bit_exact_fig1_fmaf(gpu):
     assert np.array_equal(G.view(np.uint32), oracle.gemm_nt_fmaf_f32(A, B, C0).view(np.uint32))
 
 
-@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("version", GEMM_VERSIONS)
 def test_integer_inputs_exact(gpu, version):
     # P1: integer inputs -> exact results in every version (|C| < 2^24, ints exact in TF32).
     b = 256
@@ -112,6 +113,33 @@ def test_integer_inputs_exact(gpu, version):
     assert np.array_equal(C.astype(np.int64), exact)
     (_, _, G) = _run(vs.VS_T_GEMM_NT, version, b, [A, B, C0])
     assert np.array_equal(G.astype(np.int64), C0.astype(np.int64) - A.astype(np.int64) @ B.astype(np.int64).T)
+
+
+@pytest.mark.parametrize("ttype", ["MATMUL", "GEMM_NT"])
+def test_tc_3xf16_row_scaling(gpu, ttype):
+    # R30: the split form scales each operand row (B: column for MATMUL) by its own power of
+    # two; rows spanning 2^-60 .. 2^60, an all-zero row and a row of subnormal-range fp16
+    # values (relative to the row maximum) must keep the 3xTF32-class accuracy,
+    # componentwise against |A| |B| (no overflow / underflow from fp16's range).
+    b = 256
+    rng = np.random.default_rng(5)
+    A = vsgen.uniform(700, b, b) * np.exp2(rng.integers(-60, 60, size=(b, 1))).astype(np.float32)
+    B = vsgen.uniform(701, b, b)
+    B = B * (np.exp2(rng.integers(-60, 60, size=(1, b))).astype(np.float32) if ttype == "MATMUL"
+             else np.exp2(rng.integers(-60, 60, size=(b, 1))).astype(np.float32))
+    A[3, :] = 0.0
+    A[5, :] = vsgen.uniform(702, 1, b)[0] * 1e-5
+    A[5, 0] = 1e4                        # one large entry: the rest of the row is < 2^-29 of the max
+    C0 = np.zeros((b, b), np.float32)
+    A, B = A.astype(np.float32), B.astype(np.float32)
+    t = getattr(vs, "VS_T_" + ttype)
+    (_, _, C) = _run(t, vs.VS_V_TC_3XF16, b, [A, B, C0])
+    Bop = B if ttype == "MATMUL" else B.T
+    ref = oracle.matmul(A, Bop, C0) if ttype == "MATMUL" else oracle.gemm_nt(A, B, C0)
+    bound = np.abs(A.astype(np.float64)) @ np.abs(Bop.astype(np.float64))
+    err = np.abs(C.astype(np.float64) - ref)
+    assert np.all(err <= 3e-5 * bound + 1e-37), float(np.max(err / (bound + 1e-300)))
+    assert np.all(C[3] == 0.0)
 
 
 # ------------------------------------------------------------------ trsm / potrf

@@ -20,7 +20,7 @@ NARGS = {vs.VS_T_MATMUL: 3, vs.VS_T_GEMM_NT: 3, vs.VS_T_SYRK: 2, vs.VS_T_TRSM: 2
 
 
 def bench(ttype, version, b, streams=1, iters=20):
-    dt = torch.float64 if version >= vs.VS_V_DFMA_F64 else torch.float32
+    dt = torch.float64 if version in (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64) else torch.float32
     sets = []
     for s in range(streams):
         args = [torch.randn(b, b, dtype=dt, device="cuda") * 0.1 for _ in range(NARGS[ttype])]
@@ -31,10 +31,26 @@ def bench(ttype, version, b, streams=1, iters=20):
         sets.append(args)
     strs = [torch.cuda.Stream() for _ in range(streams)]
     info = torch.zeros(1, dtype=torch.int32, device="cuda")
+    # operands in the version's derived forms, built once (as the runtime caches them)
+    ptrs = []
+    keep = []
+    for s in range(streams):
+        p = []
+        for i, t in enumerate(sets[s]):
+            f = vs.vs_operand_form(ttype, version, i)
+            if f > 0:
+                buf = torch.empty(vs.vs_form_bytes(f, b), dtype=torch.uint8, device="cuda")
+                vs.vs_form_make(f, b, t.data_ptr(), buf.data_ptr(), torch.cuda.current_stream().cuda_stream)
+                keep.append(buf)
+                p.append(buf.data_ptr())
+            else:
+                p.append(t.data_ptr())
+        ptrs.append(p)
+    torch.cuda.synchronize()
 
     def run():
         for s in range(streams):
-            vs.vs_tile_run(ttype, version, b, [t.data_ptr() for t in sets[s]], info.data_ptr(), strs[s].cuda_stream)
+            vs.vs_tile_run_prepared(ttype, version, b, ptrs[s], info.data_ptr(), strs[s].cuda_stream)
 
     for _ in range(3):
         run()
