@@ -345,6 +345,7 @@ def main():
     ap.add_argument("--small", action="store_true", help="cfg1/cfg2-sized smoke of the bench itself")
     ap.add_argument("--only", choices=["mm", "ch", "both"], default="both")
     ap.add_argument("--dump-log", default="")
+    ap.add_argument("--dump-cold-log", default="", help="decision log of the first (learning) step")
     ap.add_argument("--table-dump", default="", help="write the learned TaskVersionSets after warm-up")
     ap.add_argument("--table-load", default="", help="warm start from a table (NEXT-2 hints)")
     ap.add_argument("--replay", action="store_true", help="decisions from the loaded table (profiling runs)")
@@ -410,6 +411,8 @@ def main():
     wl.step(step_barrier)
     barrier()
     cold_ms = (time.perf_counter() - t0) * 1e3
+    if args.dump_cold_log and rank == 0:
+        json.dump({"log": rt.vs_decision_log(), "groups": rt.vs_group_stats()}, open(args.dump_cold_log, "w"))
     for _ in range(args.warmup - 1):
         wl.step(step_barrier)
     if args.table_dump:

@@ -17,27 +17,37 @@
 //   kind::f16 runs at twice the tf32 rate, so the 3-product scheme has twice the
 //   tensor-pipe ceiling of 3xTF32.
 //
-// Byte layout (Rp = R rounded up to 256, rows >= R are zero; K a multiple of 64):
-//   for each k-block kb of 64 columns: [big: Rp rows x 128 B][small: Rp rows x 128 B], each
-//   part in the UMMA canonical K-major SWIZZLE_128B layout (8-row atoms of 1024 B, 16-byte
-//   chunk index XOR (row & 7)); after the Rp*K*4 bytes: float inv_scale[Rp] = 2^-e_r.
-//   A 128-row slice of one part for one k-block is therefore one contiguous 16 KB block, so
-//   the GEMM feeds shared memory with plain bulk copies (cp.async.bulk, the TMA engine's 1-D
-//   mode): no tensor map, no register traffic, no per-task conversion.
+// Byte layout (Rp = R rounded up to 256, rows >= R are zero; K a multiple of 32):
+//   for each k-block kb of 32 columns and each group of 256 rows: [big: 256 rows x 64 B]
+//   [small: 256 rows x 64 B], each part in the UMMA canonical K-major SWIZZLE_64B layout
+//   (8-row atoms of 512 B, 16-byte chunk index XOR ((row >> 1) & 3)); after the Rp*K*4
+//   bytes: float inv_scale[Rp] = 2^-e_r, then Rp words of scratch (column maxima of
+//   split_cols).  The big+small pair of a 256-row group for one k-block is one contiguous
+//   32 KB block, so the GEMM feeds shared memory with two plain bulk copies per stage
+//   (cp.async.bulk, the TMA engine's 1-D mode; measured on B200: a bulk copy costs ~250
+//   clk of TMA issue, so 16 KB copies cap at 66 B/clk/SM and 32 KB copies reach the
+//   ~125 B/clk/SM ceiling): no tensor map, no register traffic, no per-task conversion.
 //
-// GEMM structure (one 128 x 256 output tile per CTA, cta_group::1, UMMA M=128, N=256):
-//   warp 0      lane 0 issues the bulk copies of a stage (A big/small 16 KB each, B
-//               big/small 32 KB each) onto the stage's full barrier (expect_tx).
-//   warp 1      TMEM allocator (512 columns) + MMA issuer: 4 k-steps x 3 MMAs per stage,
-//               tcgen05.commit -> empty[s]; after the last stage -> acc_full.
-//   warps 2-9   C_in staged into TMEM columns [256, 512) during the main loop; epilogue:
-//               tcgen05.ld acc and C_in, C = C_in + acc * 2^-eA(i) * 2^-eB(j), vector stores.
-// LOWER (syrk): CTAs strictly above the diagonal exit; diagonal tiles store only j <= i.
+// GEMM structure: one 256 x 256 output tile per CTA (cta_group::1), two UMMA M=128 N=256
+// accumulators in TMEM (columns [0,256) = rows 0-127, [256,512) = rows 128-255).  Per
+// 32-wide k-block a CTA stages 64 KB (A and B' big/small, 256 rows each) for 12 MMAs:
+// ~40 B/clk of L2->SM traffic at the MMA rate, vs 64 B/clk for a 128 x 256 tile — the
+// L2 (~8 TB/s measured on the 128 x 256 kernel) is what bounds this GEMM on B200.
+//   warp 0      lane 0: the bulk copies of each stage (2 x 32 KB) onto the stage's full
+//               barrier (expect_tx).
+//   warp 1      TMEM allocator (512 columns) + MMA issuer: 2 k-steps x 2 row halves x 3
+//               products per stage, tcgen05.commit -> empty[s]; last stage -> acc_full.
+//   warps 2-9   epilogue (TMEM lane quarter = warp % 4, column half = (warp - 2) / 4): per
+//               accumulator, tcgen05.ld 32-column chunks -> padded per-warp smem block (the
+//               stage buffers are free once acc_full fired), then row by row coalesced:
+//               C = C_in + acc * 2^-eA(i) * 2^-eB(j) in fp32 round-to-nearest (C_in read
+//               from global here; each epilogue thread prefetches its C row into L2 at
+//               kernel start).
+// LOWER (syrk): tiles strictly above the diagonal exit; diagonal tiles store only j <= i.
 #pragma once
 #include <cuda_fp16.h>
 #include <cuda_runtime.h>
 #include <stdint.h>
-#include <stdlib.h>
 
 #include "kernels.hpp"
 #include "task_ctx.cuh"
@@ -57,26 +67,47 @@ using tc::tc_fence_before;
 using tc::tmem_ld32;
 using tc::tmem_st32;
 
-constexpr int BM = 128, BN = 256, BK = 64;   // BK in fp16 elements (one 128-byte swizzled row)
-constexpr int STAGES = 2;
-constexpr int A_BYTES = BM * BK * 2;          // 16 KB per part
-constexpr int B_BYTES = BN * BK * 2;          // 32 KB per part
-constexpr int STAGE = 2 * A_BYTES + 2 * B_BYTES;
+// Optional per-CTA phase timeline (tools/probe_tcf.cu builds with -DVS_TCF_TRACE).
+#ifdef VS_TCF_TRACE
+__device__ unsigned long long g_tcf_trace[1024][12];
+#define TCF_T(i) g_tcf_trace[blockIdx.y * gridDim.x + blockIdx.x][i] = tc_now()
+#define TCF_ADD(i, v) g_tcf_trace[blockIdx.y * gridDim.x + blockIdx.x][i] += (v)
+__device__ __forceinline__ unsigned long long tc_now()
+{
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+    return t;
+}
+#else
+#define TCF_T(i)
+#define TCF_ADD(i, v)
+#endif
+
+constexpr int BT = 256, BK = 32;   // CTA tile 256 x 256; BK in fp16 elements (one 64-byte swizzled row)
+constexpr int STAGES = 3;
+constexpr int PART = BT * BK * 2;             // 16 KB: one part (big or small) of 256 rows
+constexpr int STAGE = 4 * PART;               // A big, A small, B big, B small
 constexpr int NEPI = 256;                     // epilogue threads (warps 2-9)
 constexpr int NTHREADS = 64 + NEPI;
+constexpr int EPI_LD = 132;                   // padded row (floats) of the epilogue staging
 constexpr int SMEM = STAGES * STAGE + 1024 /*align*/ + 256 /*barriers*/;
+static_assert(8 * 32 * EPI_LD * 4 <= STAGES * STAGE, "epilogue staging must fit in the stage buffers");
 
 __host__ __device__ inline int split_rows_padded(int R) { return (R + 255) / 256 * 256; }
 __host__ __device__ inline size_t split_bytes(int R, int K)
 {
     const size_t Rp = (size_t)split_rows_padded(R);
-    return Rp * (size_t)K * 4 + Rp * 4;
+    return Rp * (size_t)K * 4 + Rp * 8;
 }
-// byte offset of the 16-byte chunk holding elements (r, 8c .. 8c+7) of the big part
+// byte offset of the 16-byte chunk holding elements (r, 8c .. 8c+7) of the big part; the
+// small part of the same chunk is SPLIT_HALF bytes further (big and small of one 256-row
+// group are adjacent, so one 32 KB bulk copy moves both)
+constexpr int SPLIT_HALF = 256 * 64;
 __host__ __device__ inline size_t split_chunk_off(int Rp, int r, int c)
 {
-    const int kb = c >> 3, kc = c & 7;
-    return (size_t)kb * Rp * 256 + (size_t)(r >> 3) * 1024 + (r & 7) * 128 + ((kc ^ (r & 7)) << 4);
+    const int kb = c >> 2, kc = c & 3;
+    return (size_t)kb * Rp * 128 + (size_t)(r >> 8) * (2 * SPLIT_HALF) + (size_t)(r & 255) * 64 +
+           ((kc ^ ((r >> 1) & 3)) << 4);
 }
 
 // Row scale exponent: max * 2^e in [2^14, 2^15).
@@ -129,7 +160,7 @@ __global__ void __launch_bounds__(256) split_rows_kernel(const float *__restrict
     }
     const int e = row_exponent(m);
     const float sc = ldexpf(1.f, e);
-    const size_t half = (size_t)Rp * 128;
+    const size_t half = SPLIT_HALF;
     for (int k = 8 * lane; k < K; k += 256) {
         float v[8] = {0.f, 0.f, 0.f, 0.f, 0.f, 0.f, 0.f, 0.f};
         if (r < R) {
@@ -147,52 +178,57 @@ __global__ void __launch_bounds__(256) split_rows_kernel(const float *__restrict
 }
 
 // Row form of X^T for a K x R row-major fp32 matrix X (ld): form row r = column r of X.
-// One CTA per 32 columns: pass 1 = column maxima, pass 2 = 64 x 32 blocks transposed
-// through shared memory, 16-byte stores of 8 consecutive k per thread.
-__global__ void __launch_bounds__(256) split_cols_kernel(const float *__restrict__ X, int K, int R, int ld,
-                                                         uint8_t *__restrict__ out)
+// Pass 1 (split_colmax_kernel, grid (Rp/32, K/128)): column maxima of |x| folded into the
+// form's scratch words with atomicMax on the float bits (non-negative floats order as
+// integers; the scratch is zeroed first).  Pass 2 (split_cols_kernel, grid (Rp/32, K/64)):
+// 64 x 32 blocks transposed through shared memory, 16-byte stores of 8 consecutive k.
+__global__ void __launch_bounds__(256) split_colmax_kernel(const float *__restrict__ X, int K, int R, int ld,
+                                                           uint8_t *__restrict__ out)
 {
-    __shared__ float tile[64][33];
     __shared__ float cmax[8][32];
-    __shared__ int cexp[32];
     const int Rp = split_rows_padded(R);
-    const int r0 = blockIdx.x * 32, w = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int col = r0 + lane;
+    const int w = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int col = blockIdx.x * 32 + lane, k0 = blockIdx.y * 128;
     float m = 0.f;
     if (col < R)
-        for (int k = w; k < K; k += 8) m = fmaxf(m, fabsf(__ldg(X + (int64_t)k * ld + col)));
+#pragma unroll 4
+        for (int k = k0 + w; k < min(K, k0 + 128); k += 8) m = fmaxf(m, fabsf(__ldg(X + (int64_t)k * ld + col)));
     cmax[w][lane] = m;
     __syncthreads();
     if (w == 0) {
         float mm = cmax[0][lane];
 #pragma unroll
         for (int i = 1; i < 8; i++) mm = fmaxf(mm, cmax[i][lane]);
-        const int e = row_exponent(mm);
-        cexp[lane] = e;
-        if (col < Rp) reinterpret_cast<float *>(out + (size_t)Rp * K * 4)[col] = ldexpf(1.f, -e);
+        if (col < Rp) atomicMax(reinterpret_cast<int *>(out + (size_t)Rp * K * 4 + (size_t)Rp * 4) + col, __float_as_int(mm));
     }
-    __syncthreads();
-    const size_t half = (size_t)Rp * 128;
+}
+
+__global__ void __launch_bounds__(256) split_cols_kernel(const float *__restrict__ X, int K, int R, int ld,
+                                                         uint8_t *__restrict__ out)
+{
+    __shared__ float tile[64][33];
+    const int Rp = split_rows_padded(R);
+    const int r0 = blockIdx.x * 32, k0 = blockIdx.y * 64, w = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int col = r0 + lane;
+#pragma unroll
+    for (int i = 0; i < 8; i++) {
+        const int k = k0 + w * 8 + i;
+        tile[w * 8 + i][lane] = (col < R && k < K) ? __ldg(X + (int64_t)k * ld + col) : 0.f;
+    }
     const int rr = threadIdx.x >> 3, kc = threadIdx.x & 7;   // form row r0+rr, chunk kc of the block
-    const float sc = ldexpf(1.f, cexp[rr]);
-    for (int k0 = 0; k0 < K; k0 += 64) {
+    const float m = __int_as_float(reinterpret_cast<const int *>(out + (size_t)Rp * K * 4 + (size_t)Rp * 4)[r0 + rr]);
+    const int e = row_exponent(m);
+    if (blockIdx.y == 0 && kc == 0) reinterpret_cast<float *>(out + (size_t)Rp * K * 4)[r0 + rr] = ldexpf(1.f, -e);
+    __syncthreads();
+    if (k0 + kc * 8 < K) {
+        float v[8];
 #pragma unroll
-        for (int i = 0; i < 8; i++) {
-            const int k = k0 + w * 8 + i;
-            tile[w * 8 + i][lane] = (col < R) ? __ldg(X + (int64_t)k * ld + col) : 0.f;
-        }
-        __syncthreads();
-        if (r0 + rr < Rp) {
-            float v[8];
-#pragma unroll
-            for (int i = 0; i < 8; i++) v[i] = tile[kc * 8 + i][rr];
-            uint4 big, small;
-            split8(v, sc, big, small);
-            const size_t off = split_chunk_off(Rp, r0 + rr, (k0 >> 3) + kc);
-            *reinterpret_cast<uint4 *>(out + off) = big;
-            *reinterpret_cast<uint4 *>(out + off + half) = small;
-        }
-        __syncthreads();
+        for (int i = 0; i < 8; i++) v[i] = tile[kc * 8 + i][rr];
+        uint4 big, small;
+        split8(v, ldexpf(1.f, e), big, small);
+        const size_t off = split_chunk_off(Rp, r0 + rr, (k0 >> 3) + kc);
+        *reinterpret_cast<uint4 *>(out + off) = big;
+        *reinterpret_cast<uint4 *>(out + off + SPLIT_HALF) = small;
     }
 }
 
@@ -205,6 +241,23 @@ __device__ __forceinline__ void bulk_g2s(uint32_t dst, const void *src, uint32_t
     asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(dst),
                  "l"(src), "r"(bytes), "r"(smem_u32(bar))
                  : "memory");
+}
+__device__ __forceinline__ void prefetch_l2(const void *p, uint32_t bytes)
+{
+    asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(p), "r"(bytes) : "memory");
+}
+
+// UMMA shared-memory descriptor, K-major SWIZZLE_64B (layout type 4): rows of 64 B, 8-row
+// atoms of 512 B (SBO), LBO = 16 B (ignored for swizzled K-major), version 1.
+__device__ __forceinline__ uint64_t make_desc_sw64(uint32_t saddr)
+{
+    uint64_t d = 0;
+    d |= (uint64_t)((saddr & 0x3FFFF) >> 4);
+    d |= (uint64_t)(16 >> 4) << 16;
+    d |= (uint64_t)(512 >> 4) << 32;
+    d |= (uint64_t)1 << 46;
+    d |= (uint64_t)4 << 61;
+    return d;
 }
 
 // Instruction descriptor, kind::f16: D f32 (bit 4), A/B f16 (format 0), negate A (bit 13),
@@ -236,8 +289,8 @@ tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8
     uint64_t *acc_full = empty + STAGES;
     uint32_t *tmem_slot = (uint32_t *)(acc_full + 1);
 
-    const int m0 = blockIdx.y * BM, n0 = blockIdx.x * BN;
-    if (LOWER && n0 >= m0 + BM) {
+    const int m0 = blockIdx.y * BT, n0 = blockIdx.x * BT;
+    if (LOWER && n0 >= m0 + BT) {
         ctx_end(ctx);
         return;
     }
@@ -246,6 +299,7 @@ tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8
     const int RA = split_rows_padded(M), RB = split_rows_padded(N);
 
     if (threadIdx.x == 0) {
+        TCF_T(0);
         for (int s = 0; s < STAGES; s++) {
             mbar_init(&full[s], 1);
             mbar_init(&empty[s], 1);
@@ -262,6 +316,7 @@ tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8
     __syncthreads();
     tc_fence_after();
     const uint32_t tmem = *tmem_slot;
+    if (threadIdx.x == 0) TCF_T(1);
 
     if (warp == 0) {
         // ------------------------------------------------------------ bulk-copy producer
@@ -271,94 +326,122 @@ tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8
                 if (kb >= STAGES) mbar_wait(&empty[s], ((kb / STAGES) - 1) & 1);
                 const uint32_t st = smem_u32(smem + s * STAGE);
                 mbar_expect_tx(&full[s], STAGE);
-                const uint8_t *a = As + (size_t)kb * RA * 256 + (size_t)m0 * 128;
-                const uint8_t *b = Bs + (size_t)kb * RB * 256 + (size_t)n0 * 128;
-                bulk_g2s(st, a, A_BYTES, &full[s]);
-                bulk_g2s(st + A_BYTES, a + (size_t)RA * 128, A_BYTES, &full[s]);
-                bulk_g2s(st + 2 * A_BYTES, b, B_BYTES, &full[s]);
-                bulk_g2s(st + 2 * A_BYTES + B_BYTES, b + (size_t)RB * 128, B_BYTES, &full[s]);
+                bulk_g2s(st, As + (size_t)kb * RA * 128 + (size_t)m0 * 128, 2 * PART, &full[s]);
+                bulk_g2s(st + 2 * PART, Bs + (size_t)kb * RB * 128 + (size_t)n0 * 128, 2 * PART, &full[s]);
             }
         }
         __syncwarp();
     } else if (warp == 1) {
         // ------------------------------------------------------------ MMA issuer
-        constexpr uint32_t idesc = make_idesc_f16(BM, BN, NEG);
+        constexpr uint32_t idesc = make_idesc_f16(128, BT, NEG);
         for (int kb = 0; kb < nk; kb++) {
             const int s = kb % STAGES;
+#ifdef VS_TCF_TRACE
+            const unsigned long long w0 = tc_now();
+#endif
             mbar_wait(&full[s], (kb / STAGES) & 1);
+#ifdef VS_TCF_TRACE
+            if (lane == 0) {
+                TCF_ADD(9, tc_now() - w0);
+                if (kb == 0) TCF_T(2);
+                if (kb == nk / 2) TCF_T(3);
+            }
+#endif
             tc_fence_after();
             if (lane == 0) {
-                const uint32_t a_big = smem_u32(smem + s * STAGE), a_small = a_big + A_BYTES;
-                const uint32_t b_big = a_big + 2 * A_BYTES, b_small = b_big + B_BYTES;
+                const uint32_t a_big = smem_u32(smem + s * STAGE), a_small = a_big + PART;
+                const uint32_t b_big = a_big + 2 * PART, b_small = a_big + 3 * PART;
 #pragma unroll
                 for (int kk = 0; kk < BK / 16; kk++) {
-                    const uint32_t o = kk * 32;   // 16 fp16 = 32 B inside the 128 B swizzled row
-                    const uint64_t dAb = make_desc(a_big + o, 16, 1024), dAs = make_desc(a_small + o, 16, 1024);
-                    const uint64_t dBb = make_desc(b_big + o, 16, 1024), dBs = make_desc(b_small + o, 16, 1024);
-                    const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
-                    mma_f16(tmem, dAb, dBb, idesc, first);
-                    mma_f16(tmem, dAb, dBs, idesc, 1u);
-                    mma_f16(tmem, dAs, dBb, idesc, 1u);
+                    const uint32_t o = kk * 32;   // 16 fp16 = 32 B inside the 64 B swizzled row
+                    const uint64_t dBb = make_desc_sw64(b_big + o), dBs = make_desc_sw64(b_small + o);
+#pragma unroll
+                    for (int h = 0; h < 2; h++) {   // rows [128h, 128h+128) -> TMEM columns [256h, 256h+256)
+                        const uint32_t ho = h * 128 * 64;
+                        const uint64_t dAb = make_desc_sw64(a_big + ho + o), dAs = make_desc_sw64(a_small + ho + o);
+                        const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
+                        const uint32_t d = tmem + (uint32_t)(h * BT);
+                        mma_f16(d, dAb, dBb, idesc, first);
+                        mma_f16(d, dAb, dBs, idesc, 1u);
+                        mma_f16(d, dAs, dBb, idesc, 1u);
+                    }
                 }
                 tc::mma_commit(&empty[s]);
-                if (kb == nk - 1) tc::mma_commit(acc_full);
+                if (kb == nk - 1) {
+                    tc::mma_commit(acc_full);
+                    TCF_T(4);
+                }
             }
             __syncwarp();
         }
     } else {
-        // ------------------------------------------------------------ C_in staging + epilogue
-        const int eq = warp & 3, eh = (warp - 2) >> 2;   // TMEM lane quarter, column half
-        const int erow = m0 + eq * 32 + lane;
-        const float4 z4 = make_float4(0.f, 0.f, 0.f, 0.f);
-#pragma unroll 1
-        for (int c = 0; c < BN / 64; c++) {
-            const int col0 = eh * (BN / 2) + c * 32;
-            float v[32];
-            const float *crow = C + (int64_t)erow * ldc + n0 + col0;
-#pragma unroll
-            for (int j = 0; j < 8; j++) {
-                const float4 x = (erow < M && n0 + col0 + 4 * j < N) ? *reinterpret_cast<const float4 *>(crow + 4 * j) : z4;
-                v[4 * j] = x.x; v[4 * j + 1] = x.y; v[4 * j + 2] = x.z; v[4 * j + 3] = x.w;
-            }
-            tmem_st32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(BN + col0), v);
+        // ------------------------------------------------------------ epilogue
+        const int q = warp & 3, eh = (warp - 2) >> 2;   // TMEM lane quarter, column half
+        float *stg = reinterpret_cast<float *>(smem) + (warp - 2) * 32 * EPI_LD;   // this warp's 32 x 128 block
+        const int ccol = eh * 128 + lane * 4;            // this lane's 4 columns in the store phase
+        const float *sav = reinterpret_cast<const float *>(As + (size_t)RA * K * 4) + m0;
+        const float4 sb = __ldg(reinterpret_cast<const float4 *>(reinterpret_cast<const float *>(Bs + (size_t)RB * K * 4) + n0 + ccol));
+        {   // C_in into L2 while the main loop runs (LSU prefetches: bulk prefetches would
+            // occupy the TMA unit that feeds the operands): thread t -> tile row t, its 1 KB
+            const int r = threadIdx.x - 64;
+            if (m0 + r < M)
+                for (int c = 0; c < min(BT, N - n0); c += 32)
+                    asm volatile("prefetch.global.L2 [%0];" ::"l"(C + (int64_t)(m0 + r) * ldc + n0 + c));
         }
-        asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
-        const float sa = erow < RA ? __ldg(reinterpret_cast<const float *>(As + (size_t)RA * K * 4) + erow) : 0.f;
-        const float *sbv = reinterpret_cast<const float *>(Bs + (size_t)RB * K * 4) + n0;
-
+        if (warp == 2 && lane == 0) TCF_T(5);
         mbar_wait(acc_full, 0);
         tc_fence_after();
+        if (warp == 2 && lane == 0) TCF_T(6);
+        const int gcol = n0 + ccol;
 #pragma unroll 1
-        for (int c = 0; c < BN / 64; c++) {
-            const int col0 = eh * (BN / 2) + c * 32;
-            float v[32], cv[32];
-            tmem_ld32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)col0, v);
-            tmem_ld32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(BN + col0), cv);
+        for (int h = 0; h < 2; h++) {
+            const int rbase = h * 128 + q * 32;          // tile rows of this warp
+            const float sa_l = __ldg(sav + rbase + lane);
+#pragma unroll 1
+            for (int c = 0; c < 4; c++) {
+                float v[32];
+                tmem_ld32(tmem + ((uint32_t)(q * 32) << 16) + (uint32_t)(h * BT + eh * 128 + c * 32), v);
 #pragma unroll
-            for (int j = 0; j < 8; j++) {
-                const float4 sb = __ldg(reinterpret_cast<const float4 *>(sbv + col0) + j);
-                v[4 * j + 0] = cv[4 * j + 0] + (v[4 * j + 0] * sa) * sb.x;
-                v[4 * j + 1] = cv[4 * j + 1] + (v[4 * j + 1] * sa) * sb.y;
-                v[4 * j + 2] = cv[4 * j + 2] + (v[4 * j + 2] * sa) * sb.z;
-                v[4 * j + 3] = cv[4 * j + 3] + (v[4 * j + 3] * sa) * sb.w;
+                for (int j = 0; j < 8; j++)
+                    *reinterpret_cast<float4 *>(stg + lane * EPI_LD + c * 32 + 4 * j) =
+                        make_float4(v[4 * j], v[4 * j + 1], v[4 * j + 2], v[4 * j + 3]);
             }
-            if (erow < M) {
-                float *crow = C + (int64_t)erow * ldc + n0 + col0;
+            __syncwarp();
+            // 16 rows per round: all C_in loads of the round in flight before the first use
+#pragma unroll 1
+            for (int r0 = 0; r0 < 32; r0 += 16) {
+                float4 cin[16];
 #pragma unroll
-                for (int j = 0; j < 8; j++) {
-                    const int col = n0 + col0 + 4 * j;
-                    if (col >= N) break;
-                    if (LOWER && col + 3 > erow) {
-                        if (col + 0 <= erow) crow[4 * j + 0] = v[4 * j + 0];
-                        if (col + 1 <= erow) crow[4 * j + 1] = v[4 * j + 1];
-                        if (col + 2 <= erow) crow[4 * j + 2] = v[4 * j + 2];
-                    } else {
-                        *reinterpret_cast<float4 *>(crow + 4 * j) =
-                            make_float4(v[4 * j + 0], v[4 * j + 1], v[4 * j + 2], v[4 * j + 3]);
+                for (int i = 0; i < 16; i++) {
+                    const int grow = m0 + rbase + r0 + i;
+                    cin[i] = (grow < M && gcol < N) ? *reinterpret_cast<const float4 *>(C + (int64_t)grow * ldc + gcol)
+                                                    : make_float4(0.f, 0.f, 0.f, 0.f);
+                }
+#pragma unroll
+                for (int i = 0; i < 16; i++) {
+                    const int r = r0 + i, grow = m0 + rbase + r;
+                    const float sa = __shfl_sync(0xffffffffu, sa_l, r);
+                    if (grow < M && gcol < N) {
+                        float *cp = C + (int64_t)grow * ldc + gcol;
+                        const float4 a = *reinterpret_cast<const float4 *>(stg + r * EPI_LD + lane * 4);
+                        float4 o;
+                        o.x = cin[i].x + (a.x * sa) * sb.x;
+                        o.y = cin[i].y + (a.y * sa) * sb.y;
+                        o.z = cin[i].z + (a.z * sa) * sb.z;
+                        o.w = cin[i].w + (a.w * sa) * sb.w;
+                        if (LOWER && gcol + 3 > grow) {
+                            if (gcol + 0 <= grow) cp[0] = o.x;
+                            if (gcol + 1 <= grow) cp[1] = o.y;
+                            if (gcol + 2 <= grow) cp[2] = o.z;
+                        } else {
+                            *reinterpret_cast<float4 *>(cp) = o;
+                        }
                     }
                 }
             }
+            __syncwarp();
         }
+        if (warp == 2 && lane == 0) TCF_T(8);
     }
 
     tc_fence_before();
@@ -370,230 +453,11 @@ tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8
     ctx_end(ctx);
 }
 
-// ---------------------------------------------------------------- CTA-pair variant
-// A cluster of two CTAs computes a 256 x 256 output tile with UMMA M=256, N=256
-// (cta_group::2): CTA r stages rows [128r, 128r+128) of A and rows [128r, 128r+128) of the
-// pair's B' slice in ITS shared memory (bulk copies onto its own full[s]); a relay thread
-// of each CTA then arrives on the LEADER's pfull[s] (count 2); the leader issues the MMAs,
-// which read both CTAs' operands, and tcgen05.commit multicasts empty[s] to both CTAs.
-// Per SM and per 64-wide k-block this stages 64 KB (vs 96 KB for one CTA at 128 x 256):
-// 42 B/clk of L2 traffic at the MMA rate instead of 64 (the L2 delivers ~42 B/clk/SM).
-constexpr int P_STAGES = 3;
-constexpr int P_A_BYTES = 128 * BK * 2;    // 16 KB per part (this CTA's 128 rows of A)
-constexpr int P_B_BYTES = 128 * BK * 2;    // 16 KB per part (this CTA's 128 rows of B')
-constexpr int P_STAGE = 2 * P_A_BYTES + 2 * P_B_BYTES;
-constexpr int P_SMEM = P_STAGES * P_STAGE + 1024 + 256;
-
-__device__ __forceinline__ uint32_t cluster_rank()
-{
-    uint32_t r;
-    asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(r));
-    return r;
-}
-__device__ __forceinline__ void cluster_sync()
-{
-    asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
-}
-__device__ __forceinline__ void mbar_arrive_cluster(uint64_t *bar, uint32_t target)
-{
-    uint32_t remote;
-    asm volatile("mapa.shared::cluster.u32 %0, %1, %2;" : "=r"(remote) : "r"(smem_u32(bar)), "r"(target));
-    asm volatile("mbarrier.arrive.release.cluster.shared::cluster.b64 _, [%0];" ::"r"(remote) : "memory");
-}
-__device__ __forceinline__ void mbar_wait_cluster(uint64_t *bar, uint32_t parity)
-{
-    asm volatile(
-        "{\n\t.reg .pred P1;\n"
-        "WAIT_%=:\n\t"
-        "mbarrier.try_wait.parity.acquire.cluster.shared::cta.b64 P1, [%0], %1;\n\t"
-        "@P1 bra DONE_%=;\n\t"
-        "bra WAIT_%=;\n"
-        "DONE_%=:\n\t}" ::"r"(smem_u32(bar)),
-        "r"(parity)
-        : "memory");
-}
-__device__ __forceinline__ void mma_f16_pair(uint32_t tmem_d, uint64_t adesc, uint64_t bdesc, uint32_t idesc, uint32_t acc)
-{
-    asm volatile(
-        "{\n\t.reg .pred p;\n\t"
-        "setp.ne.b32 p, %4, 0;\n\t"
-        "tcgen05.mma.cta_group::2.kind::f16 [%0], %1, %2, %3, p;\n\t}" ::"r"(tmem_d),
-        "l"(adesc), "l"(bdesc), "r"(idesc), "r"(acc));
-}
-__device__ __forceinline__ void mma_commit_pair(uint64_t *bar)
-{
-    asm volatile(
-        "tcgen05.commit.cta_group::2.mbarrier::arrive::one.shared::cluster.multicast::cluster.b64 [%0], %1;" ::"r"(
-            smem_u32(bar)),
-        "h"((uint16_t)0x3)
-        : "memory");
-}
-
-template <bool NEG, bool LOWER>
-__global__ void __cluster_dims__(2, 1, 1) __launch_bounds__(NTHREADS, 1)
-tcf_gemm2_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8_t *__restrict__ Bs,
-                 float *__restrict__ C, int ldc, TaskCtx ctx)
-{
-    ctx_begin(ctx);
-    extern __shared__ uint8_t smem_raw[];
-    uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
-    uint64_t *full = (uint64_t *)(smem + P_STAGES * P_STAGE);
-    uint64_t *pfull = full + P_STAGES;
-    uint64_t *empty = pfull + P_STAGES;
-    uint64_t *acc_full = empty + P_STAGES;
-    uint32_t *tmem_slot = (uint32_t *)(acc_full + 1);
-
-    const uint32_t crank = cluster_rank();
-    const int pair_m0 = (blockIdx.x & ~1) * 128;
-    const int m0 = pair_m0 + (int)crank * 128;
-    const int n0 = blockIdx.y * 256;
-    const int nb0 = n0 + (int)crank * 128;
-    if (LOWER && n0 >= pair_m0 + 256) {
-        ctx_end(ctx);
-        return;
-    }
-    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int nk = K / BK;
-    const int RA = split_rows_padded(M), RB = split_rows_padded(N);
-
-    if (threadIdx.x == 0) {
-        for (int s = 0; s < P_STAGES; s++) {
-            mbar_init(&full[s], 1);
-            mbar_init(&pfull[s], 2);
-            mbar_init(&empty[s], 1);
-        }
-        mbar_init(acc_full, 1);
-        asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-    }
-    if (warp == 1) {
-        asm volatile("tcgen05.alloc.cta_group::2.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(tmem_slot)),
-                     "r"(512u));
-        asm volatile("tcgen05.relinquish_alloc_permit.cta_group::2.sync.aligned;");
-    }
-    tc_fence_before();
-    cluster_sync();
-    tc_fence_after();
-    const uint32_t tmem = *tmem_slot;
-
-    if (warp == 0) {
-        // ------------------------------------------------------------ bulk-copy producer
-        if (lane == 0) {
-            for (int kb = 0; kb < nk; kb++) {
-                const int s = kb % P_STAGES;
-                if (kb >= P_STAGES) mbar_wait(&empty[s], ((kb / P_STAGES) - 1) & 1);
-                const uint32_t st = smem_u32(smem + s * P_STAGE);
-                mbar_expect_tx(&full[s], P_STAGE);
-                const uint8_t *a = As + (size_t)kb * RA * 256 + (size_t)m0 * 128;
-                const uint8_t *b = Bs + (size_t)kb * RB * 256 + (size_t)nb0 * 128;
-                bulk_g2s(st, a, P_A_BYTES, &full[s]);
-                bulk_g2s(st + P_A_BYTES, a + (size_t)RA * 128, P_A_BYTES, &full[s]);
-                bulk_g2s(st + 2 * P_A_BYTES, b, P_B_BYTES, &full[s]);
-                bulk_g2s(st + 2 * P_A_BYTES + P_B_BYTES, b + (size_t)RB * 128, P_B_BYTES, &full[s]);
-            }
-        }
-        __syncwarp();
-    } else if (warp == 1) {
-        // ------------------------------------------------------------ relay (+ MMA issue in the leader)
-        constexpr uint32_t idesc = make_idesc_f16(256, 256, NEG);
-        for (int kb = 0; kb < nk; kb++) {
-            const int s = kb % P_STAGES;
-            const uint32_t par = (kb / P_STAGES) & 1;
-            if (lane == 0) {
-                mbar_wait(&full[s], par);            // this CTA's operands landed
-                mbar_arrive_cluster(&pfull[s], 0);   // tell the leader
-            }
-            if (crank == 0) {
-                mbar_wait_cluster(&pfull[s], par);   // both CTAs' operands landed
-                tc_fence_after();
-                if (lane == 0) {
-                    const uint32_t a_big = smem_u32(smem + s * P_STAGE), a_small = a_big + P_A_BYTES;
-                    const uint32_t b_big = a_big + 2 * P_A_BYTES, b_small = b_big + P_B_BYTES;
-#pragma unroll
-                    for (int kk = 0; kk < BK / 16; kk++) {
-                        const uint32_t o = kk * 32;
-                        const uint64_t dAb = make_desc(a_big + o, 16, 1024), dAs = make_desc(a_small + o, 16, 1024);
-                        const uint64_t dBb = make_desc(b_big + o, 16, 1024), dBs = make_desc(b_small + o, 16, 1024);
-                        const uint32_t first = (kb == 0 && kk == 0) ? 0u : 1u;
-                        mma_f16_pair(tmem, dAb, dBb, idesc, first);
-                        mma_f16_pair(tmem, dAb, dBs, idesc, 1u);
-                        mma_f16_pair(tmem, dAs, dBb, idesc, 1u);
-                    }
-                    mma_commit_pair(&empty[s]);
-                    if (kb == nk - 1) mma_commit_pair(acc_full);
-                }
-            }
-            __syncwarp();
-        }
-    } else {
-        // ------------------------------------------------------------ C_in staging + epilogue
-        const int eq = warp & 3, eh = (warp - 2) >> 2;
-        const int erow = m0 + eq * 32 + lane;
-        const float4 z4 = make_float4(0.f, 0.f, 0.f, 0.f);
-#pragma unroll 1
-        for (int c = 0; c < 4; c++) {
-            const int col0 = eh * 128 + c * 32;
-            float v[32];
-            const float *crow = C + (int64_t)erow * ldc + n0 + col0;
-#pragma unroll
-            for (int j = 0; j < 8; j++) {
-                const float4 x = (erow < M && n0 + col0 + 4 * j < N) ? *reinterpret_cast<const float4 *>(crow + 4 * j) : z4;
-                v[4 * j] = x.x; v[4 * j + 1] = x.y; v[4 * j + 2] = x.z; v[4 * j + 3] = x.w;
-            }
-            tmem_st32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(256 + col0), v);
-        }
-        asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory");
-        const float sa = __ldg(reinterpret_cast<const float *>(As + (size_t)RA * K * 4) + erow);
-        const float *sbv = reinterpret_cast<const float *>(Bs + (size_t)RB * K * 4) + n0;
-
-        mbar_wait(acc_full, 0);
-        tc_fence_after();
-#pragma unroll 1
-        for (int c = 0; c < 4; c++) {
-            const int col0 = eh * 128 + c * 32;
-            float v[32], cv[32];
-            tmem_ld32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)col0, v);
-            tmem_ld32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(256 + col0), cv);
-#pragma unroll
-            for (int j = 0; j < 8; j++) {
-                const float4 sb = __ldg(reinterpret_cast<const float4 *>(sbv + col0) + j);
-                v[4 * j + 0] = cv[4 * j + 0] + (v[4 * j + 0] * sa) * sb.x;
-                v[4 * j + 1] = cv[4 * j + 1] + (v[4 * j + 1] * sa) * sb.y;
-                v[4 * j + 2] = cv[4 * j + 2] + (v[4 * j + 2] * sa) * sb.z;
-                v[4 * j + 3] = cv[4 * j + 3] + (v[4 * j + 3] * sa) * sb.w;
-            }
-            if (erow < M) {
-                float *crow = C + (int64_t)erow * ldc + n0 + col0;
-#pragma unroll
-                for (int j = 0; j < 8; j++) {
-                    const int col = n0 + col0 + 4 * j;
-                    if (col >= N) break;
-                    if (LOWER && col + 3 > erow) {
-                        if (col + 0 <= erow) crow[4 * j + 0] = v[4 * j + 0];
-                        if (col + 1 <= erow) crow[4 * j + 1] = v[4 * j + 1];
-                        if (col + 2 <= erow) crow[4 * j + 2] = v[4 * j + 2];
-                    } else {
-                        *reinterpret_cast<float4 *>(crow + 4 * j) =
-                            make_float4(v[4 * j + 0], v[4 * j + 1], v[4 * j + 2], v[4 * j + 3]);
-                    }
-                }
-            }
-        }
-    }
-
-    tc_fence_before();
-    cluster_sync();
-    if (warp == 1) {
-        tc_fence_after();
-        asm volatile("tcgen05.dealloc.cta_group::2.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"(512u));
-    }
-    ctx_end(ctx);
-}
-
 // ---------------------------------------------------------------- host launchers
 // Split forms: X is R x K row-major (ld) -> row form; X is K x R row-major -> row form of X^T.
 inline int split_rows(const float *X, int R, int K, int ld, void *out, cudaStream_t s)
 {
-    if (R <= 0 || K <= 0 || K % 64 || ld % 4) return -1;
+    if (R <= 0 || K <= 0 || K % 32 || ld % 4) return -1;
     const int Rp = split_rows_padded(R);
     count_launch();
     split_rows_kernel<<<(Rp + 7) / 8, 256, 0, s>>>(X, R, K, ld, (uint8_t *)out);
@@ -601,51 +465,24 @@ inline int split_rows(const float *X, int R, int K, int ld, void *out, cudaStrea
 }
 inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStream_t s)
 {
-    if (R <= 0 || K <= 0 || K % 64) return -1;
+    if (R <= 0 || K <= 0 || K % 32) return -1;
     const int Rp = split_rows_padded(R);
+    if (cudaMemsetAsync((uint8_t *)out + (size_t)Rp * K * 4 + (size_t)Rp * 4, 0, (size_t)Rp * 4, s) != cudaSuccess)
+        return -1;
     count_launch();
-    split_cols_kernel<<<Rp / 32, 256, 0, s>>>(X, K, R, ld, (uint8_t *)out);
+    split_colmax_kernel<<<dim3(Rp / 32, (K + 127) / 128), 256, 0, s>>>(X, K, R, ld, (uint8_t *)out);
+    count_launch();
+    split_cols_kernel<<<dim3(Rp / 32, (K + 63) / 64), 256, 0, s>>>(X, K, R, ld, (uint8_t *)out);
     return 0;
 }
 
-// CTA-pair launcher (VS_TCF_PAIR=0 selects the single-CTA kernel).
-template <bool NEG, bool LOWER>
-inline int tcf_gemm2(int M, int N, int K, const void *As, const void *Bs, float *C, int ldc, cudaStream_t s,
-                     const TaskCtx &ctx)
-{
-    auto kern = tcf_gemm2_kernel<NEG, LOWER>;
-    static bool attr[64] = {};
-    int dev = 0;
-    cudaGetDevice(&dev);
-    if (!attr[dev & 63]) {
-        cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, P_SMEM);
-        attr[dev & 63] = true;
-    }
-    int gx = (M + 127) / 128;
-    gx += gx & 1;
-    dim3 grid(gx, (N + 255) / 256);
-    count_launch();
-    kern<<<grid, NTHREADS, P_SMEM, s>>>(M, N, K, (const uint8_t *)As, (const uint8_t *)Bs, C, ldc, ctx);
-    return 0;
-}
-
-inline bool tcf_pair_enabled()
-{
-    static int v = [] {
-        const char *e = getenv("VS_TCF_PAIR");
-        return e ? atoi(e) : 1;
-    }();
-    return v != 0;
-}
-
-// C (M x N, ldc) += s * A * B'^T with A, B' in split form (K a multiple of 64).
+// C (M x N, ldc) += s * A * B'^T with A, B' in split form (K a multiple of 32).
 template <bool NEG, bool LOWER>
 inline int tcf_gemm(int M, int N, int K, const void *As, const void *Bs, float *C, int ldc, cudaStream_t s,
                     const TaskCtx &ctx = TaskCtx())
 {
     if (M <= 0 || N <= 0) return 0;
     if (K % BK || ldc % 4) return -1;
-    if (tcf_pair_enabled()) return tcf_gemm2<NEG, LOWER>(M, N, K, As, Bs, C, ldc, s, ctx);
     auto kern = tcf_gemm_kernel<NEG, LOWER>;
     static bool attr[64] = {};
     int dev = 0;
@@ -654,7 +491,7 @@ inline int tcf_gemm(int M, int N, int K, const void *As, const void *Bs, float *
         cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
         attr[dev & 63] = true;
     }
-    dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
+    dim3 grid((N + BT - 1) / BT, (M + BT - 1) / BT);
     count_launch();
     kern<<<grid, NTHREADS, SMEM, s>>>(M, N, K, (const uint8_t *)As, (const uint8_t *)Bs, C, ldc, ctx);
     return 0;
