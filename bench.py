@@ -36,7 +36,7 @@ CH_N, CH_B = 32768, 1024
 SEED_MM, SEED_CH = 3, 4
 # runtime configuration the bench times (env VS_SLOTS / VS_PRIORITY / VS_QDEPTH override):
 # lambda 3, 6 workers (streams) per GPU, NEXT-4 bottom-level priority with queue depth 2
-RT_DEFAULTS = dict(lam=3, slots=6, priority=2, qdepth=2)
+RT_DEFAULTS = dict(lam=3, slots=6, priority=2, qdepth=2, group=8)
 F32_VERSIONS_MASK = 0b100111  # simt_f32 | tc_3xtf32 | f64in_f32io | tc_3xf16 (gemm-type tasks)
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
@@ -340,6 +340,8 @@ def main():
     ap.add_argument("--priority", type=int, default=int(os.environ.get("VS_PRIORITY", RT_DEFAULTS["priority"])))
     ap.add_argument("--qdepth", type=int, default=int(os.environ.get("VS_QDEPTH", RT_DEFAULTS["qdepth"])))
     ap.add_argument("--lam", type=int, default=RT_DEFAULTS["lam"])
+    ap.add_argument("--group", type=int, default=int(os.environ.get("VS_GROUP", RT_DEFAULTS["group"])),
+                    help="tasks per grouped launch (vs_config.group_tasks)")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--small", action="store_true", help="cfg1/cfg2-sized smoke of the bench itself")
@@ -381,7 +383,7 @@ def main():
     prio, qdepth = args.priority, args.qdepth
     look = int(os.environ.get("VS_LOOKAHEAD", "0"))
     cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0,
-                               priority=prio, lookahead=look, queue_depth=qdepth)
+                               priority=prio, lookahead=look, queue_depth=qdepth, group_tasks=args.group)
     rt = vs.Runtime(cfg)
     if world > 1:
         shm = gather("/vsched_%d_%d" % (os.getpid(), int(time.time())) if rank == 0 else None)[0]
@@ -450,7 +452,8 @@ def main():
     # ---- e2e: same step through the C ABI with HOST (pinned) buffers, copies inside the timed region
     e2e = None
     if not args.no_e2e and world == 1:
-        rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look, queue_depth=qdepth))
+        rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look,
+                                              queue_depth=qdepth, group_tasks=args.group))
         wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, with_mm=with_mm, with_ch=with_ch)
         wl2.step()     # warm-up incl. learning
         tsum, h2d, d2h = 0.0, 0, 0
@@ -503,13 +506,16 @@ def main():
             "roofline": roof,
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
             "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
-            "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "mode": "runahead"},
+            "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "group_tasks": args.group,
+                                "mode": "runahead"},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
             "operand_forms_per_step": int((st1.forms_built - st0.forms_built) / args.steps),
             "device_tx_bytes_per_step": int((st1.device_tx_bytes - st0.device_tx_bytes) / args.steps),
-            "host_us_per_task": {"decide": round((st1.host_ns_decide - st0.host_ns_decide) / 1e3 / max(1, len(log)), 3),
-                                 "issue": round((st1.host_ns_issue - st0.host_ns_issue) / 1e3 / max(1, len(log)), 3)},
+            "host_us_per_task": {k: round((getattr(st1, "host_ns_" + k) - getattr(st0, "host_ns_" + k)) / 1e3 / max(1, len(log)), 3)
+                                 for k in ("decide", "issue", "launch", "deps", "poll", "vevent", "flush")},
+            "host_idle_loops_per_task": round((st1.host_idle_loops - st0.host_idle_loops) / max(1, len(log)), 2),
+            "host_loops_per_task": round((st1.host_loops - st0.host_loops) / max(1, len(log)), 2),
         }
         print(json.dumps(out))
         if args.dump_log:

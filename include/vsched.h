@@ -142,12 +142,21 @@ typedef struct {
                           worker holds fewer than d virtual tasks (running + queued), and only
                           to such workers; the rest wait in the (priority) ready queue, so a
                           task released later on the critical path overtakes them (NEXT-4) */
+    int group_tasks;   /* grouped launches (this build): up to this many consecutive tasks of
+                          one worker whose version can share a launch (tc_3xf16 MATMUL /
+                          GEMM_NT / SYRK) are enqueued as ONE kernel launch on the worker's
+                          stream (no dependences inside a group: a task whose predecessor is
+                          still pending flushes it first).  0 or 1: one launch per task */
+    int group_wait_us; /* a pending group is launched after this many microseconds of host
+                          time even if not full (and whenever the runtime has nothing else to
+                          do); 0 = default 20 */
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,
  * run-ahead, live timing, flush.  Environment overrides applied by vs_create (L277-288):
  * VS_LAMBDA, VS_SLOTS, VS_POLICY(=versioning|fixed:<v>), VS_LEARNING(=hold|rr),
- * VS_MODE(=runahead|ready), VS_LOOKAHEAD(=n), VS_PRIORITY(=0|1|2), VS_QDEPTH(=d). */
+ * VS_MODE(=runahead|ready), VS_LOOKAHEAD(=n), VS_PRIORITY(=0|1|2), VS_QDEPTH(=d),
+ * VS_GROUP(=tasks per grouped launch), VS_GROUP_US. */
 void vs_config_default(vs_config *cfg);
 
 /* Create a runtime.  *out receives an opaque handle owning scheduler state, DAG,
@@ -226,6 +235,13 @@ typedef struct {
     int64_t tracker;          /* dependence tracker in use: 1 = device completion words
                                  (stream memory operations), 0 = CUDA events */
     int64_t forms_built;      /* derived operand forms built (VS_V_TC_3XF16 split halves) */
+    int64_t host_ns_poll;     /* host time polling device completions */
+    int64_t host_ns_launch;   /* part of host_ns_issue spent enqueuing the version's kernels */
+    int64_t host_ns_deps;     /* part of host_ns_issue spent enqueuing dependence waits / forms */
+    int64_t host_loops;       /* iterations of the runtime's drive loop */
+    int64_t host_ns_vevent;   /* host time advancing the virtual clock (run-ahead DES) */
+    int64_t host_ns_flush;    /* host time launching pending grouped launches from the loop */
+    int64_t host_idle_loops;  /* drive-loop iterations that found nothing to do */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 

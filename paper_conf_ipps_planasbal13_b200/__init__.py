@@ -41,14 +41,15 @@ class vs_config(Structure):
                 ("lambda_", c_int), ("policy", c_int), ("fixed_version", c_int), ("learning", c_int),
                 ("mode", c_int), ("replay", c_int), ("flush", c_int), ("lookahead", c_int), ("priority", c_int),
                 ("group_ratio_permille", c_int), ("ewma_weight", c_int), ("locality_gbps", c_int),
-                ("queue_depth", c_int)]
+                ("queue_depth", c_int), ("group_tasks", c_int), ("group_wait_us", c_int)]
 
 
 class vs_stats_t(Structure):
     _fields_ = [(n, c_int64) for n in (
         "tasks_submitted", "tasks_completed", "decisions", "input_tx_bytes", "output_tx_bytes", "device_tx_bytes",
         "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns",
-        "kernel_launches", "tracker", "forms_built")]
+        "kernel_launches", "tracker", "forms_built", "host_ns_poll", "host_ns_launch", "host_ns_deps", "host_loops", "host_ns_vevent", "host_ns_flush",
+        "host_idle_loops")]
 
 
 class vs_group_stat_t(Structure):

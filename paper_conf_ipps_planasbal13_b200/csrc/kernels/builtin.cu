@@ -173,6 +173,29 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
     return -1;
 }
 
+struct TaskGroup {
+    tcf::TcfGroup g;
+};
+int group_kind(int type, int version)
+{
+    return (version == VS_V_TC_3XF16 && (type == VS_T_MATMUL || type == VS_T_GEMM_NT || type == VS_T_SYRK)) ? 1 : 0;
+}
+TaskGroup *group_new() { return new TaskGroup(); }
+void group_free(TaskGroup *g) { delete g; }
+int group_size(const TaskGroup *g) { return g->g.n; }
+int group_ctas(const TaskGroup *g) { return g->g.ctas; }
+int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const TaskCtx &ctx)
+{
+    if (!group_kind(type, version)) return -1;
+    switch (type) {
+    case VS_T_MATMUL: return tcf::tcf_group_add(g->g, b, b, b, p[0], p[1], (float *)p[2], b, false, false, ctx);
+    case VS_T_GEMM_NT: return tcf::tcf_group_add(g->g, b, b, b, p[0], p[1], (float *)p[2], b, true, false, ctx);
+    case VS_T_SYRK: return tcf::tcf_group_add(g->g, b, b, b, p[0], p[0], (float *)p[1], b, true, true, ctx);
+    }
+    return -1;
+}
+int group_launch(TaskGroup *g, cudaStream_t s) { return tcf::tcf_group_launch(g->g, s); }
+
 namespace {
 // tc_3xf16: p[] holds the split forms of the in-operands (builtin_operand_form)
 int run_f16(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)

@@ -17,11 +17,13 @@ inline std::atomic<long long> &launch_counter()
 inline void count_launch() { launch_counter().fetch_add(1, std::memory_order_relaxed); }
 
 // Per-task execution record passed to every kernel of a built-in version (task_ctx.cuh).
-// slot: device memory {start_min, end_max, ticket}; host: host-mapped {start, end}.
+// slot: device memory {start_min, end_max, ticket}; host: host-mapped {start, end,
+// kernels completed, pad}.
 // A default TaskCtx (nullptrs) disables recording (direct vs_tile_run calls).
 struct TaskCtx {
     unsigned long long *slot = nullptr;
     unsigned long long *host = nullptr;
+    unsigned int ncta = 0;   // CTAs of the task in the launch (0: the whole grid)
 };
 
 // Task types / versions use the VS_T_* / VS_V_* numbering of vsched.h.
@@ -39,6 +41,20 @@ int builtin_operand_form(int type, int version, int param);
 size_t form_bytes(int form, int b);
 // Build the form of the b x b fp32 tile src into dst (form_bytes) on stream s.
 int make_form(int form, int b, const void *src, void *dst, cudaStream_t s);
+
+// Grouped launches: versions whose tasks can share one kernel launch with other tasks of
+// the same kind (tc_3xf16 MATMUL / GEMM_NT / SYRK: one grouped tcgen05 GEMM launch).
+// group_kind() = 0 for versions that cannot be grouped.  A group is filled with
+// group_add() (ptrs as for launch_builtin, ctx of the task; returns the task's CTA count,
+// or -1 if it does not fit / is unsupported) and launched by group_launch().
+struct TaskGroup;
+int group_kind(int type, int version);
+TaskGroup *group_new();
+void group_free(TaskGroup *g);
+int group_size(const TaskGroup *g);
+int group_ctas(const TaskGroup *g);
+int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const TaskCtx &ctx);
+int group_launch(TaskGroup *g, cudaStream_t s);   // launches and empties the group
 
 int gen_uniform(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b, void *out,
                 cudaStream_t s);

@@ -39,7 +39,8 @@ __device__ __forceinline__ void ctx_end(const TaskCtx &c)
     if (threadIdx.x == 0) {
         __threadfence();
         atomicMax(&c.slot[1], globaltimer_ns());
-        const unsigned long long nct = (unsigned long long)gridDim.x * gridDim.y * gridDim.z;
+        const unsigned long long nct = c.ncta ? (unsigned long long)c.ncta
+                                              : (unsigned long long)gridDim.x * gridDim.y * gridDim.z;
         if (atomicAdd(&c.slot[2], 1ull) == nct - 1) {
             __threadfence();
             const unsigned long long s = atomicAdd(&c.slot[0], 0ull), e = atomicAdd(&c.slot[1], 0ull);
@@ -47,6 +48,10 @@ __device__ __forceinline__ void ctx_end(const TaskCtx &c)
                 volatile unsigned long long *h = c.host;
                 h[0] = s;
                 h[1] = e;
+                // kernels of the task completed so far: the host polls this word (compared
+                // with the number of kernels the version launched) instead of querying events
+                __threadfence_system();
+                h[2] = h[2] + 1;
             }
             atomicExch(&c.slot[2], 0ull);   // re-arm for the task's next kernel
         }

@@ -276,12 +276,25 @@ __device__ __forceinline__ void mma_f16(uint32_t tmem_d, uint64_t adesc, uint64_
         "l"(adesc), "l"(bdesc), "r"(idesc), "r"(acc));
 }
 
-template <bool NEG, bool LOWER>
-__global__ void __launch_bounds__(NTHREADS, 1)
-tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8_t *__restrict__ Bs,
-                float *__restrict__ C, int ldc, TaskCtx ctx)
+// One GEMM task of a grouped launch: C (M x N, ldc) += s * A * B'^T on split forms.
+// flags: bit 0 = negate (s = -1), bit 1 = LOWER (only tiles with j <= i exist, and the
+// diagonal tiles store j <= i).  The task's CTAs are [tile0, tile0 + ntiles) of the grid.
+struct TcfTask {
+    const uint8_t *As, *Bs;
+    float *C;
+    int M, N, K, ldc;
+    int flags, tile0, ntiles, tiles_n;
+    TaskCtx ctx;
+};
+constexpr int kMaxGroup = 24;
+struct TcfGroup {
+    int n = 0, ctas = 0;
+    TcfTask t[kMaxGroup];
+};
+static_assert(sizeof(TcfGroup) <= 4000, "kernel parameter space");
+
+__global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_constant__ TcfGroup grp)
 {
-    ctx_begin(ctx);
     extern __shared__ uint8_t smem_raw[];
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     uint64_t *full = (uint64_t *)(smem + STAGES * STAGE);
@@ -289,11 +302,29 @@ tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8
     uint64_t *acc_full = empty + STAGES;
     uint32_t *tmem_slot = (uint32_t *)(acc_full + 1);
 
-    const int m0 = blockIdx.y * BT, n0 = blockIdx.x * BT;
-    if (LOWER && n0 >= m0 + BT) {
-        ctx_end(ctx);
-        return;
+    // this CTA's task and output tile
+    int ti = 0;
+    while (ti + 1 < grp.n && (int)blockIdx.x >= grp.t[ti + 1].tile0) ti++;
+    const TcfTask &tk = grp.t[ti];
+    const TaskCtx ctx = tk.ctx;
+    ctx_begin(ctx);
+    const int M = tk.M, N = tk.N, K = tk.K, ldc = tk.ldc;
+    const uint8_t *__restrict__ As = tk.As;
+    const uint8_t *__restrict__ Bs = tk.Bs;
+    float *__restrict__ C = tk.C;
+    const bool NEG = tk.flags & 1, LOWER = (tk.flags >> 1) & 1;
+    const int l = (int)blockIdx.x - tk.tile0;
+    int bi, bj;
+    if (LOWER) {   // l = bi (bi + 1) / 2 + bj, bj <= bi
+        bi = (int)((sqrtf(8.f * l + 1.f) - 1.f) * 0.5f);
+        while ((bi + 1) * (bi + 2) / 2 <= l) bi++;
+        while (bi * (bi + 1) / 2 > l) bi--;
+        bj = l - bi * (bi + 1) / 2;
+    } else {
+        bi = l / tk.tiles_n;
+        bj = l % tk.tiles_n;
     }
+    const int m0 = bi * BT, n0 = bj * BT;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int nk = K / BK;
     const int RA = split_rows_padded(M), RB = split_rows_padded(N);
@@ -333,7 +364,7 @@ tcf_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ As, const uint8
         __syncwarp();
     } else if (warp == 1) {
         // ------------------------------------------------------------ MMA issuer
-        constexpr uint32_t idesc = make_idesc_f16(128, BT, NEG);
+        const uint32_t idesc = make_idesc_f16(128, BT, NEG);
         for (int kb = 0; kb < nk; kb++) {
             const int s = kb % STAGES;
 #ifdef VS_TCF_TRACE
@@ -476,25 +507,55 @@ inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStrea
     return 0;
 }
 
-// C (M x N, ldc) += s * A * B'^T with A, B' in split form (K a multiple of 32).
-template <bool NEG, bool LOWER>
-inline int tcf_gemm(int M, int N, int K, const void *As, const void *Bs, float *C, int ldc, cudaStream_t s,
-                    const TaskCtx &ctx = TaskCtx())
+// Append one task to a group; returns its CTA count, 0 for an empty task, -1 if it does
+// not fit or is unsupported (K a multiple of 32, ldc of 4).
+inline int tcf_group_add(TcfGroup &g, int M, int N, int K, const void *As, const void *Bs, float *C, int ldc,
+                         bool neg, bool lower, TaskCtx ctx)
 {
     if (M <= 0 || N <= 0) return 0;
-    if (K % BK || ldc % 4) return -1;
-    auto kern = tcf_gemm_kernel<NEG, LOWER>;
+    if (K % BK || ldc % 4 || g.n >= kMaxGroup || (lower && M != N)) return -1;
+    const int tm = (M + BT - 1) / BT, tn = (N + BT - 1) / BT;
+    const int nt = lower ? tm * (tm + 1) / 2 : tm * tn;
+    TcfTask &t = g.t[g.n++];
+    t.As = (const uint8_t *)As;
+    t.Bs = (const uint8_t *)Bs;
+    t.C = C;
+    t.M = M; t.N = N; t.K = K; t.ldc = ldc;
+    t.flags = (neg ? 1 : 0) | (lower ? 2 : 0);
+    t.tile0 = g.ctas;
+    t.ntiles = nt;
+    t.tiles_n = tn;
+    ctx.ncta = (unsigned)nt;
+    t.ctx = ctx;
+    g.ctas += nt;
+    return nt;
+}
+
+inline int tcf_group_launch(TcfGroup &g, cudaStream_t s)
+{
+    if (g.n == 0) return 0;
     static bool attr[64] = {};
     int dev = 0;
     cudaGetDevice(&dev);
     if (!attr[dev & 63]) {
-        cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
         attr[dev & 63] = true;
     }
-    dim3 grid((N + BT - 1) / BT, (M + BT - 1) / BT);
     count_launch();
-    kern<<<grid, NTHREADS, SMEM, s>>>(M, N, K, (const uint8_t *)As, (const uint8_t *)Bs, C, ldc, ctx);
+    tcf_gemm_kernel<<<g.ctas, NTHREADS, SMEM, s>>>(g);
+    g.n = g.ctas = 0;
     return 0;
+}
+
+// C (M x N, ldc) += s * A * B'^T with A, B' in split form (K a multiple of 32): one task.
+template <bool NEG, bool LOWER>
+inline int tcf_gemm(int M, int N, int K, const void *As, const void *Bs, float *C, int ldc, cudaStream_t s,
+                    const TaskCtx &ctx = TaskCtx())
+{
+    TcfGroup g;
+    const int r = tcf_group_add(g, M, N, K, As, Bs, C, ldc, NEG, LOWER, ctx);
+    if (r <= 0) return r;
+    return tcf_group_launch(g, s);
 }
 
 }  // namespace tcf
