@@ -519,7 +519,7 @@ def main():
         }
         print(json.dumps(out))
         if args.dump_log:
-            json.dump({"log": log, "groups": groups}, open(args.dump_log, "w"))
+            json.dump({"log": log, "groups": groups, "issue": rt.vs_decision_issue_ns()}, open(args.dump_log, "w"))
     barrier()
     rt.close()
     if dist is not None:

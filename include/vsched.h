@@ -273,6 +273,11 @@ typedef struct {
     int64_t t_start_ns, t_end_ns; /* sim: virtual clock; gpu: GPU timeline of the version's
                                      start/end events (ns since runtime creation) */
 } vs_decision_t;
+/* Host wall-clock time at which each decision-log entry's task was enqueued on its
+ * stream, on the t_start_ns timeline (system clock minus the same origin: the GPU's
+ * %globaltimer follows the host's system clock); 0 if not issued (sim).  Same indexing
+ * and (cap, n) protocol as vs_decision_log.  Diagnostic. */
+int vs_decision_issue_ns(vs_rt rt, int64_t *out, int64_t cap, int64_t *n);
 /* Copy up to cap records (from the beginning) into out; *n = total records. */
 int vs_decision_log(vs_rt rt, vs_decision_t *out, int64_t cap, int64_t *n);
 /* FNV-1a 64 over (task, version, worker, t_decide) of every record, little-endian int64

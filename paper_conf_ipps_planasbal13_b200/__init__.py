@@ -127,6 +127,7 @@ def lib():
         "vs_form_bytes": (c_int64, [c_int, c_int]),
         "vs_form_make": (c_int, [c_int, c_int, c_void_p, c_void_p, c_void_p]),
         "vs_tile_run_prepared": (c_int, [c_int, c_int, c_int, POINTER(c_void_p), c_void_p, c_void_p]),
+        "vs_decision_issue_ns": (c_int, [rt, POINTER(c_int64), c_int64, POINTER(c_int64)]),
     }
     for name, (res, args) in sig.items():
         f = getattr(L, name)
@@ -143,7 +144,7 @@ EXPORTED = ["vs_config_default", "vs_create", "vs_destroy", "vs_last_error", "vs
             "vs_replay_set", "vs_app_matmul", "vs_app_cholesky", "vs_tile_run", "vs_gen_uniform", "vs_gen_spd",
             "vs_build_info", "vs_gen_tile", "vs_dist_init", "vs_data_set_owner", "vs_ipc_export", "vs_ipc_open",
             "vs_ipc_close", "vs_data_invalidate", "vs_operand_form", "vs_form_bytes", "vs_form_make",
-            "vs_tile_run_prepared"]
+            "vs_tile_run_prepared", "vs_decision_issue_ns"]
 
 
 def _ids(seq, ctype=c_int64):
@@ -336,6 +337,13 @@ class Runtime:
         lib().vs_decision_log(self.h, buf, n.value, ctypes.byref(n))
         return [(r.task, r.version, r.worker, r.t_decide_ns, r.t_start_ns, r.t_end_ns, r.phase, r.type)
                 for r in buf[:n.value]]
+
+    def vs_decision_issue_ns(self):
+        n = c_int64()
+        lib().vs_decision_issue_ns(self.h, None, 0, ctypes.byref(n))
+        buf = (c_int64 * max(1, n.value))()
+        lib().vs_decision_issue_ns(self.h, buf, n.value, ctypes.byref(n))
+        return list(buf[:n.value])
 
     def vs_decision_log_hash(self) -> int:
         return int(lib().vs_decision_log_hash(self.h))
