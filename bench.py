@@ -35,8 +35,9 @@ MM_N, MM_B = 16384, 1024
 CH_N, CH_B = 32768, 1024
 SEED_MM, SEED_CH = 3, 4
 # runtime configuration the bench times (env VS_SLOTS / VS_PRIORITY / VS_QDEPTH override):
-# lambda 3, 6 workers (streams) per GPU, NEXT-4 bottom-level priority with queue depth 2
-RT_DEFAULTS = dict(lam=3, slots=6, priority=2, qdepth=2, group=8)
+# lambda 3, 4 workers (streams) per GPU, NEXT-4 bottom-level priority with queue depth 2,
+# grouped launches of up to 8 tc_3xf16 tasks
+RT_DEFAULTS = dict(lam=3, slots=4, priority=2, qdepth=2, group=8)
 F32_VERSIONS_MASK = 0b100111  # simt_f32 | tc_3xtf32 | f64in_f32io | tc_3xf16 (gemm-type tasks)
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731

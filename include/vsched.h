@@ -97,7 +97,8 @@ enum {
     VS_V_DFMA_F64 = 3,    /* fp64 tiles, SIMT DFMA */
     VS_V_DMMA_F64 = 4,    /* fp64 tiles, mma.sync f64 tensor cores */
     VS_V_TC_3XF16 = 5,    /* fp32 tiles, tcgen05 kind::f16 on row-scaled fp16 big/small halves of the
-                             operands (reading R30); MATMUL, GEMM_NT and SYRK only.  Its in-operands
+                             operands (reading R30); MATMUL, GEMM_NT, SYRK, and TRSM as X = B inv(L)^T
+                             (R31); no POTRF.  Its in-operands
                              are read through a per-GPU cached "split form" that the runtime builds
                              (one conversion kernel per datum version, like a tile move) */
     VS_NUM_BUILTIN_VERSIONS = 6
@@ -315,12 +316,16 @@ int vs_tile_run(int type, int version, int b, void *const *ptrs, int *dinfo, voi
 
 /* Derived operand forms (reading R30).  vs_operand_form returns the form (0 = the tile
  * itself, 1 = row split form, 2 = column split form, i.e. the row split form of the
- * transposed tile) in which `version` reads parameter `param` of built-in `type`;
+ * transposed tile, 3 = row split form of inv(L)) in which `version` reads parameter `param`
+ * of built-in `type`;
  * vs_form_bytes the size of a form of a b x b fp32 tile (0 for form 0).
  * vs_form_make enqueues the conversion of the b x b fp32 tile `src` into `dst`
  * (vs_form_bytes bytes, device memory, 16-byte aligned) on `stream`.
- * vs_tile_run_prepared is vs_tile_run with ptrs[param] already in its form (no
- * conversion): the kernel the runtime launches for a task.  VS_E_INVAL on bad arguments. */
+ * vs_tile_run_prepared is vs_tile_run with the forms prepared by the caller (no
+ * conversion): ptrs holds 2 * nparams pointers, ptrs[i] = the tile of parameter i (device),
+ * ptrs[nparams + i] = its form (ignored for form 0) — the kernels the runtime launches for a
+ * task.  Form 3 (TRSM of VS_V_TC_3XF16) = row split form of inv(L) for the lower triangle L
+ * of the tile (reading R31).  VS_E_INVAL on bad arguments. */
 int vs_operand_form(int type, int version, int param);
 int64_t vs_form_bytes(int form, int b);
 int vs_form_make(int form, int b, const void *src, void *dst, void *stream);

@@ -9,7 +9,8 @@
 //   f64in_f32io    fp32     dmma_gemm<float>  (DMMA on upcast operands)            blocked
 //   dfma_f64       fp64     simt_gemm<double,double> (DFMA)                        blocked
 //   dmma_f64       fp64     dmma_gemm<double>  (mma.sync f64)                      blocked
-//   tc_3xf16       fp32     tcf_gemm (tcgen05 kind::f16 on split forms, tc_f16.cuh) (gemm types only)
+//   tc_3xf16       fp32     tcf_gemm (tcgen05 kind::f16 on split forms, tc_f16.cuh); TRSM = GEMM with
+//                           the inv(L) form (R31); no potrf
 //
 // potrf of tc_3xtf32 is the single-launch left-looking tc_panel kernel (tc_panel.cuh).
 // potrf of the other versions is recursive: potrf(A11); A21 <- A21 L11^{-T} (trsm);
@@ -148,9 +149,15 @@ bool builtin_supported(int type, int version, int b)
 {
     if (type < 0 || type >= VS_NUM_BUILTIN_TYPES) return false;
     if (version < 0 || version >= VS_NUM_BUILTIN_VERSIONS) return false;
-    if (version == VS_V_TC_3XF16 && (type == VS_T_POTRF || type == VS_T_TRSM)) return false;
+    if (version == VS_V_TC_3XF16 && type == VS_T_POTRF) return false;
     if (b && (b % 64 != 0 || b < 64 || b > 4096)) return false;
     return true;
+}
+
+int builtin_nparams(int type)
+{
+    static const int np[VS_NUM_BUILTIN_TYPES] = {3, 1, 2, 2, 3};
+    return (type >= 0 && type < VS_NUM_BUILTIN_TYPES) ? np[type] : 0;
 }
 
 int builtin_operand_form(int type, int version, int param)
@@ -160,16 +167,31 @@ int builtin_operand_form(int type, int version, int param)
     case VS_T_MATMUL: return param == 0 ? FORM_SPLIT_ROWS : param == 1 ? FORM_SPLIT_COLS : FORM_RAW;
     case VS_T_GEMM_NT: return param <= 1 ? FORM_SPLIT_ROWS : FORM_RAW;
     case VS_T_SYRK: return param == 0 ? FORM_SPLIT_ROWS : FORM_RAW;
+    case VS_T_TRSM: return param == 0 ? FORM_INV_L : param == 1 ? FORM_SPLIT_ROWS : FORM_RAW;   // X = B inv(L)^T
     }
     return FORM_RAW;
 }
 
-size_t form_bytes(int form, int b) { return form == FORM_RAW ? 0 : tcf::split_bytes(b, b); }
+size_t form_bytes(int form, int b)
+{
+    if (form == FORM_RAW) return 0;
+    const size_t sb = (tcf::split_bytes(b, b) + 255) / 256 * 256;
+    return form == FORM_INV_L ? sb + (size_t)b * b * 4 : sb;   // + fp32 scratch for inv(L)^T
+}
 
 int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
 {
     if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
     if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
+    if (form == FORM_INV_L) {
+        // X = I L^{-T} by the substitution kernel of tc_3xtf32 (tc_panel), then the row
+        // split form of X^T = inv(L): reading R31 (TRSM of tc_3xf16 multiplies by it)
+        float *X = (float *)((uint8_t *)dst + (tcf::split_bytes(b, b) + 255) / 256 * 256);
+        count_launch();
+        tcf::eye_kernel<<<148, 256, 0, s>>>(X, b);
+        if (tc::tc_trsm(b, b, (const float *)src, b, X, b, s)) return -1;
+        return tcf::split_cols(X, b, b, b, dst, s);
+    }
     return -1;
 }
 
@@ -178,7 +200,7 @@ struct TaskGroup {
 };
 int group_kind(int type, int version)
 {
-    return (version == VS_V_TC_3XF16 && (type == VS_T_MATMUL || type == VS_T_GEMM_NT || type == VS_T_SYRK)) ? 1 : 0;
+    return (version == VS_V_TC_3XF16 && type != VS_T_POTRF) ? 1 : 0;
 }
 TaskGroup *group_new() { return new TaskGroup(); }
 void group_free(TaskGroup *g) { delete g; }
@@ -187,10 +209,11 @@ int group_ctas(const TaskGroup *g) { return g->g.ctas; }
 int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const TaskCtx &ctx)
 {
     if (!group_kind(type, version)) return -1;
-    switch (type) {
-    case VS_T_MATMUL: return tcf::tcf_group_add(g->g, b, b, b, p[0], p[1], (float *)p[2], b, false, false, ctx);
-    case VS_T_GEMM_NT: return tcf::tcf_group_add(g->g, b, b, b, p[0], p[1], (float *)p[2], b, true, false, ctx);
-    case VS_T_SYRK: return tcf::tcf_group_add(g->g, b, b, b, p[0], p[0], (float *)p[1], b, true, true, ctx);
+    switch (type) {   // p[i] tiles, p[np + i] forms (np = 3 / 2 / 2)
+    case VS_T_MATMUL: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, false, false, ctx);
+    case VS_T_GEMM_NT: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, true, false, ctx);
+    case VS_T_SYRK: return tcf::tcf_group_add(g->g, b, b, b, p[2], p[2], (float *)p[1], b, true, true, ctx);
+    case VS_T_TRSM: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[2], (float *)p[1], b, false, false, ctx, true);
     }
     return -1;
 }
@@ -200,12 +223,10 @@ namespace {
 // tc_3xf16: p[] holds the split forms of the in-operands (builtin_operand_form)
 int run_f16(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
 {
-    switch (type) {
-    case VS_T_MATMUL: return tcf::tcf_gemm<false, false>(b, b, b, p[0], p[1], (float *)p[2], b, s, ctx);
-    case VS_T_GEMM_NT: return tcf::tcf_gemm<true, false>(b, b, b, p[0], p[1], (float *)p[2], b, s, ctx);
-    case VS_T_SYRK: return tcf::tcf_gemm<true, true>(b, b, b, p[0], p[0], (float *)p[1], b, s, ctx);
-    }
-    return -1;
+    TaskGroup g;
+    const int r = group_add(&g, type, VS_V_TC_3XF16, b, p, ctx);
+    if (r <= 0) return r;
+    return group_launch(&g, s);
 }
 }  // namespace
 

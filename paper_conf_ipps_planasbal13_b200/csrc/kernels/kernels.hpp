@@ -21,9 +21,10 @@ inline void count_launch() { launch_counter().fetch_add(1, std::memory_order_rel
 // kernels completed, pad}.
 // A default TaskCtx (nullptrs) disables recording (direct vs_tile_run calls).
 struct TaskCtx {
-    unsigned long long *slot = nullptr;
-    unsigned long long *host = nullptr;
+    unsigned long long *slot = nullptr;   // device {~start min, end max, CTA ticket, CTA busy sum, longest CTA, -}
+    unsigned long long *host = nullptr;   // host-mapped {~start, end, kernels done, exec time}
     unsigned int ncta = 0;   // CTAs of the task in the launch (0: the whole grid)
+    unsigned int nsm = 0;    // SMs of the device (CTAs that can run at once, 1 per SM)
 };
 
 // Task types / versions use the VS_T_* / VS_V_* numbering of vsched.h.
@@ -36,7 +37,11 @@ int builtin_elem_bytes(int version);
 
 // Operand forms: a version may read an in-parameter through a derived copy of the tile
 // that the runtime builds and caches per (datum version, GPU), like a replica (a8).
-enum { FORM_RAW = 0, FORM_SPLIT_ROWS = 1, FORM_SPLIT_COLS = 2, NUM_FORMS = 3 };
+// FORM_INV_L: row split form of inv(L) for the lower triangle L of a tile (TRSM by GEMM).
+// Pointer layout of launch_builtin / group_add for versions with forms: p[i] = the tile
+// of parameter i, p[nparams + i] = its form (nparams = builtin_nparams(type)).
+enum { FORM_RAW = 0, FORM_SPLIT_ROWS = 1, FORM_SPLIT_COLS = 2, FORM_INV_L = 3, NUM_FORMS = 4 };
+int builtin_nparams(int type);
 int builtin_operand_form(int type, int version, int param);
 size_t form_bytes(int form, int b);
 // Build the form of the b x b fp32 tile src into dst (form_bytes) on stream s.

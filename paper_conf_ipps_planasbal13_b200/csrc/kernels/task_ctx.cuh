@@ -24,10 +24,21 @@ __device__ __forceinline__ unsigned long long globaltimer_ns()
     return t;
 }
 
+// start of this CTA (thread 0), for its busy time
+__device__ __forceinline__ unsigned long long &ctx_cta_start()
+{
+    __shared__ unsigned long long t0;
+    return t0;
+}
+
 __device__ __forceinline__ void ctx_begin(const TaskCtx &c)
 {
     // slot[0] keeps ~start so that max(~t) == min(t) and an all-zero slot is "empty"
-    if (c.slot && threadIdx.x == 0) atomicMax(&c.slot[0], ~globaltimer_ns());
+    if (c.slot && threadIdx.x == 0) {
+        const unsigned long long t = globaltimer_ns();
+        ctx_cta_start() = t;
+        atomicMax(&c.slot[0], ~t);
+    }
 }
 
 // Call once per CTA, by all threads of the CTA, on every exit path (after the CTA's
@@ -38,16 +49,24 @@ __device__ __forceinline__ void ctx_end(const TaskCtx &c)
     __syncthreads();
     if (threadIdx.x == 0) {
         __threadfence();
-        atomicMax(&c.slot[1], globaltimer_ns());
+        const unsigned long long t = globaltimer_ns();
+        atomicMax(&c.slot[1], t);
+        const unsigned long long dur = t - ctx_cta_start();
+        atomicAdd(&c.slot[3], dur);   // CTA busy time
+        atomicMax(&c.slot[4], dur);   // longest CTA
         const unsigned long long nct = c.ncta ? (unsigned long long)c.ncta
                                               : (unsigned long long)gridDim.x * gridDim.y * gridDim.z;
         if (atomicAdd(&c.slot[2], 1ull) == nct - 1) {
             __threadfence();
             const unsigned long long s = atomicAdd(&c.slot[0], 0ull), e = atomicAdd(&c.slot[1], 0ull);
+            const unsigned long long busy = atomicExch(&c.slot[3], 0ull), longest = atomicExch(&c.slot[4], 0ull);
             if (c.host) {
                 volatile unsigned long long *h = c.host;
                 h[0] = s;
                 h[1] = e;
+                // the kernel's execution time with the GPU to itself (reading R17): its
+                // longest CTA when all CTAs fit at once (one per SM), else CTA busy time / SMs
+                h[3] = h[3] + ((c.nsm && nct > c.nsm) ? busy / c.nsm : longest);
                 // kernels of the task completed so far: the host polls this word (compared
                 // with the number of kernels the version launched) instead of querying events
                 __threadfence_system();

@@ -278,7 +278,7 @@ __device__ __forceinline__ void mma_f16(uint32_t tmem_d, uint64_t adesc, uint64_
 
 // One GEMM task of a grouped launch: C (M x N, ldc) += s * A * B'^T on split forms.
 // flags: bit 0 = negate (s = -1), bit 1 = LOWER (only tiles with j <= i exist, and the
-// diagonal tiles store j <= i).  The task's CTAs are [tile0, tile0 + ntiles) of the grid.
+// diagonal tiles store j <= i), bit 2 = BETA0 (C = s A B'^T: C_in is not read).  The task's CTAs are [tile0, tile0 + ntiles) of the grid.
 struct TcfTask {
     const uint8_t *As, *Bs;
     float *C;
@@ -412,8 +412,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         const int ccol = eh * 128 + lane * 4;            // this lane's 4 columns in the store phase
         const float *sav = reinterpret_cast<const float *>(As + (size_t)RA * K * 4) + m0;
         const float4 sb = __ldg(reinterpret_cast<const float4 *>(reinterpret_cast<const float *>(Bs + (size_t)RB * K * 4) + n0 + ccol));
-        {   // C_in into L2 while the main loop runs (LSU prefetches: bulk prefetches would
-            // occupy the TMA unit that feeds the operands): thread t -> tile row t, its 1 KB
+        const bool BETA0 = (tk.flags >> 2) & 1;   // C = s A B'^T (C_in not read)
+        if (!BETA0) {   // C_in into L2 while the main loop runs (LSU prefetches: bulk prefetches
+            // would occupy the TMA unit that feeds the operands): thread t -> tile row t, its 1 KB
             const int r = threadIdx.x - 64;
             if (m0 + r < M)
                 for (int c = 0; c < min(BT, N - n0); c += 32)
@@ -445,8 +446,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
 #pragma unroll
                 for (int i = 0; i < 16; i++) {
                     const int grow = m0 + rbase + r0 + i;
-                    cin[i] = (grow < M && gcol < N) ? *reinterpret_cast<const float4 *>(C + (int64_t)grow * ldc + gcol)
-                                                    : make_float4(0.f, 0.f, 0.f, 0.f);
+                    cin[i] = (!BETA0 && grow < M && gcol < N) ? *reinterpret_cast<const float4 *>(C + (int64_t)grow * ldc + gcol)
+                                                              : make_float4(0.f, 0.f, 0.f, 0.f);
                 }
 #pragma unroll
                 for (int i = 0; i < 16; i++) {
@@ -510,7 +511,7 @@ inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStrea
 // Append one task to a group; returns its CTA count, 0 for an empty task, -1 if it does
 // not fit or is unsupported (K a multiple of 32, ldc of 4).
 inline int tcf_group_add(TcfGroup &g, int M, int N, int K, const void *As, const void *Bs, float *C, int ldc,
-                         bool neg, bool lower, TaskCtx ctx)
+                         bool neg, bool lower, TaskCtx ctx, bool beta0 = false)
 {
     if (M <= 0 || N <= 0) return 0;
     if (K % BK || ldc % 4 || g.n >= kMaxGroup || (lower && M != N)) return -1;
@@ -521,7 +522,7 @@ inline int tcf_group_add(TcfGroup &g, int M, int N, int K, const void *As, const
     t.Bs = (const uint8_t *)Bs;
     t.C = C;
     t.M = M; t.N = N; t.K = K; t.ldc = ldc;
-    t.flags = (neg ? 1 : 0) | (lower ? 2 : 0);
+    t.flags = (neg ? 1 : 0) | (lower ? 2 : 0) | (beta0 ? 4 : 0);
     t.tile0 = g.ctas;
     t.ntiles = nt;
     t.tiles_n = tn;
@@ -545,6 +546,12 @@ inline int tcf_group_launch(TcfGroup &g, cudaStream_t s)
     tcf_gemm_kernel<<<g.ctas, NTHREADS, SMEM, s>>>(g);
     g.n = g.ctas = 0;
     return 0;
+}
+
+__global__ void eye_kernel(float *X, int n)
+{
+    for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < (int64_t)n * n; i += (int64_t)gridDim.x * blockDim.x)
+        X[i] = (i / n == i % n) ? 1.f : 0.f;
 }
 
 // C (M x N, ldc) += s * A * B'^T with A, B' in split form (K a multiple of 32): one task.

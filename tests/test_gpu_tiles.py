@@ -143,7 +143,7 @@ def test_tc_3xf16_row_scaling(gpu, ttype):
 
 
 # ------------------------------------------------------------------ trsm / potrf
-@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("version", F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS)
 @pytest.mark.parametrize("b", [64, 128, 192, 512])
 def test_trsm_tile(gpu, version, b):
     dt = _dt(version)

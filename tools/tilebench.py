@@ -35,17 +35,18 @@ def bench(ttype, version, b, streams=1, iters=20):
     ptrs = []
     keep = []
     for s in range(streams):
-        p = []
+        p = [t.data_ptr() for t in sets[s]]
+        fp = []
         for i, t in enumerate(sets[s]):
             f = vs.vs_operand_form(ttype, version, i)
             if f > 0:
                 buf = torch.empty(vs.vs_form_bytes(f, b), dtype=torch.uint8, device="cuda")
                 vs.vs_form_make(f, b, t.data_ptr(), buf.data_ptr(), torch.cuda.current_stream().cuda_stream)
                 keep.append(buf)
-                p.append(buf.data_ptr())
+                fp.append(buf.data_ptr())
             else:
-                p.append(t.data_ptr())
-        ptrs.append(p)
+                fp.append(0)
+        ptrs.append(p + fp)
     torch.cuda.synchronize()
 
     def run():
