@@ -30,14 +30,20 @@ import time
 
 ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
+# the runtime drives ~2 x slots + 3 streams per GPU; with the default 8 hardware work
+# queues several streams share one and a critical-path launch waits behind another
+# stream's queued work (must be set before the CUDA context exists)
+os.environ.setdefault("CUDA_DEVICE_MAX_CONNECTIONS", "32")
 
 MM_N, MM_B = 16384, 1024
 CH_N, CH_B = 32768, 1024
 SEED_MM, SEED_CH = 3, 4
 # runtime configuration the bench times (env VS_SLOTS / VS_PRIORITY / VS_QDEPTH override):
-# lambda 3, 4 workers (streams) per GPU, NEXT-4 bottom-level priority with queue depth 2,
-# grouped launches of up to 8 tc_3xf16 tasks
-RT_DEFAULTS = dict(lam=3, slots=4, priority=2, qdepth=2, group=8)
+# lambda 3, 8 workers (streams) per GPU, decisions when predecessors completed (ready mode:
+# no cross-stream waits, so no stream is blocked at its head), NEXT-4 bottom-level priority
+# with a real queue cap of 2 grouped launches per worker, grouped launches of up to 8
+# tc_3xf16 tasks, critical-path tasks on their own greatest-priority streams
+RT_DEFAULTS = dict(lam=3, slots=8, priority=2, qdepth=2, group=8, mode="ready")
 F32_VERSIONS_MASK = 0b100111  # simt_f32 | tc_3xtf32 | f64in_f32io | tc_3xf16 (gemm-type tasks)
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
@@ -341,6 +347,8 @@ def main():
     ap.add_argument("--priority", type=int, default=int(os.environ.get("VS_PRIORITY", RT_DEFAULTS["priority"])))
     ap.add_argument("--qdepth", type=int, default=int(os.environ.get("VS_QDEPTH", RT_DEFAULTS["qdepth"])))
     ap.add_argument("--lam", type=int, default=RT_DEFAULTS["lam"])
+    ap.add_argument("--mode", choices=["ready", "runahead"], default=os.environ.get("VS_MODE", RT_DEFAULTS["mode"]),
+                    help="decide when predecessors completed (ready) or on the virtual clock (runahead)")
     ap.add_argument("--group", type=int, default=int(os.environ.get("VS_GROUP", RT_DEFAULTS["group"])),
                     help="tasks per grouped launch (vs_config.group_tasks)")
     ap.add_argument("--no-e2e", action="store_true")
@@ -383,8 +391,9 @@ def main():
     # in the bench; --priority 0 --qdepth 0 reproduces the paper-literal rule (R15)
     prio, qdepth = args.priority, args.qdepth
     look = int(os.environ.get("VS_LOOKAHEAD", "0"))
+    mode = 1 if args.mode == "ready" else 0          # VS_MODE_READY / VS_MODE_RUNAHEAD
     cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0,
-                               priority=prio, lookahead=look, queue_depth=qdepth, group_tasks=args.group)
+                               priority=prio, lookahead=look, queue_depth=qdepth, group_tasks=args.group, mode=mode)
     rt = vs.Runtime(cfg)
     if world > 1:
         shm = gather("/vsched_%d_%d" % (os.getpid(), int(time.time())) if rank == 0 else None)[0]
@@ -454,7 +463,7 @@ def main():
     e2e = None
     if not args.no_e2e and world == 1:
         rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look,
-                                              queue_depth=qdepth, group_tasks=args.group))
+                                              queue_depth=qdepth, group_tasks=args.group, mode=mode))
         wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, with_mm=with_mm, with_ch=with_ch)
         wl2.step()     # warm-up incl. learning
         tsum, h2d, d2h = 0.0, 0, 0
@@ -508,7 +517,7 @@ def main():
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
             "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
             "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "group_tasks": args.group,
-                                "mode": "runahead"},
+                                "mode": args.mode, "cuda_device_max_connections": os.environ.get("CUDA_DEVICE_MAX_CONNECTIONS")},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
             "operand_forms_per_step": int((st1.forms_built - st0.forms_built) / args.steps),

@@ -139,10 +139,11 @@ typedef struct {
                           (locality-aware versioning, future work L978-984; NEXT-1) */
     int queue_depth;   /* 0: a ready task is assigned at once to its earliest executor,
                           whatever that worker's queue holds (paper, L414-422).  d > 0
-                          (run-ahead and SIM only): a ready task is assigned only while some
-                          worker holds fewer than d virtual tasks (running + queued), and only
-                          to such workers; the rest wait in the (priority) ready queue, so a
-                          task released later on the critical path overtakes them (NEXT-4) */
+                          (run-ahead, SIM): a ready task is assigned only while some worker
+                          holds fewer than d virtual tasks (running + queued), and only to such
+                          workers; (ready mode): fewer than d x group_tasks issued, unfinished
+                          tasks.  The rest wait in the (priority) ready queue, so a task
+                          released later on the critical path overtakes them (NEXT-4) */
     int group_tasks;   /* grouped launches (this build): up to this many consecutive tasks of
                           one worker whose version can share a launch (tc_3xf16 MATMUL /
                           GEMM_NT / SYRK) are enqueued as ONE kernel launch on the worker's

@@ -19,18 +19,21 @@ def cholesky_ids(nt):
     return out
 
 
-def main(path, nt=32):
+def main(path, nt=32, offset=0, per_step=None):
+    """offset: tasks submitted before the Cholesky in each step (4096 matmul tasks in the
+    default bench step); per_step: tasks per step (default: the Cholesky's alone)."""
     d = json.load(open(path))
     log = d["log"]
     iss = d.get("issue") or [0] * len(log)
     log = [list(r) + [iss[n]] for n, r in enumerate(log)]
     ids = cholesky_ids(nt)
-    per = len(ids)
+    per = per_step or (len(ids) + offset)
     tmin = min(r[0] for r in log)
     by = {}
     for r in log:
-        step = (r[0] - tmin) // per
-        by.setdefault(step, {})[(r[0] - tmin) % per] = r
+        step, pos = (r[0] - tmin) // per, (r[0] - tmin) % per - offset
+        if pos >= 0:
+            by.setdefault(step, {})[pos] = r
     rs = by[max(by)]
     t0 = min(r[4] for r in rs.values())
     idx = {x: n for n, x in enumerate(ids)}
@@ -54,4 +57,4 @@ def main(path, nt=32):
 
 
 if __name__ == "__main__":
-    main(sys.argv[1])
+    main(sys.argv[1], offset=int(sys.argv[2]) if len(sys.argv) > 2 else 0)
