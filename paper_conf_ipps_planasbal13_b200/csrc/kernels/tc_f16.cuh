@@ -287,13 +287,19 @@ struct TcfTask {
     TaskCtx ctx;
 };
 constexpr int kMaxGroup = 24;
-struct TcfGroup {
+// host-side accumulator of a grouped launch; the kernel receives a copy sized to the group
+// (TcfGroupN<G>, G = 1, 4 or kMaxGroup): kernel parameters are copied by the launch, and a
+// 2 KB parameter block costs host launch time on every single-task launch
+template <int G>
+struct TcfGroupN {
     int n = 0, ctas = 0;
-    TcfTask t[kMaxGroup];
+    TcfTask t[G];
 };
+using TcfGroup = TcfGroupN<kMaxGroup>;
 static_assert(sizeof(TcfGroup) <= 4000, "kernel parameter space");
 
-__global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_constant__ TcfGroup grp)
+template <int G>
+__global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_constant__ TcfGroupN<G> grp)
 {
     extern __shared__ uint8_t smem_raw[];
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
@@ -539,11 +545,24 @@ inline int tcf_group_launch(TcfGroup &g, cudaStream_t s)
     int dev = 0;
     cudaGetDevice(&dev);
     if (!attr[dev & 63]) {
-        cudaFuncSetAttribute(tcf_gemm_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<kMaxGroup>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
         attr[dev & 63] = true;
     }
     count_launch();
-    tcf_gemm_kernel<<<g.ctas, NTHREADS, SMEM, s>>>(g);
+    if (g.n == 1) {
+        TcfGroupN<1> h;
+        h.n = 1; h.ctas = g.ctas; h.t[0] = g.t[0];
+        tcf_gemm_kernel<1><<<g.ctas, NTHREADS, SMEM, s>>>(h);
+    } else if (g.n <= 4) {
+        TcfGroupN<4> h;
+        h.n = g.n; h.ctas = g.ctas;
+        for (int i = 0; i < g.n; i++) h.t[i] = g.t[i];
+        tcf_gemm_kernel<4><<<g.ctas, NTHREADS, SMEM, s>>>(h);
+    } else {
+        tcf_gemm_kernel<kMaxGroup><<<g.ctas, NTHREADS, SMEM, s>>>(g);
+    }
     g.n = g.ctas = 0;
     return 0;
 }
