@@ -39,14 +39,25 @@ MM_N, MM_B = 16384, 1024
 CH_N, CH_B = 32768, 1024
 SEED_MM, SEED_CH = 3, 4
 # runtime configuration the bench times (env VS_SLOTS / VS_PRIORITY / VS_QDEPTH override):
-# lambda 3, 8 workers (streams) per GPU, decisions when predecessors completed (ready mode:
+# lambda 3, 12 workers (streams) per GPU, decisions when predecessors completed (ready mode:
 # no cross-stream waits, so no stream is blocked at its head), NEXT-4 bottom-level priority
 # with a real queue cap of 2 grouped launches per worker, grouped launches of up to 8
-# tc_3xf16 tasks, critical-path tasks on their own greatest-priority streams
-RT_DEFAULTS = dict(lam=3, slots=8, priority=2, qdepth=2, group=8, mode="ready")
+# tc_3xf16 tasks held up to 200 us while their stream still runs a kernel (group_hold),
+# critical-path tasks on their own greatest-priority streams
+RT_DEFAULTS = dict(lam=3, slots=12, priority=2, qdepth=2, group=8, mode="ready", hold=1, group_us=200)
 F32_VERSIONS_MASK = 0b100111  # simt_f32 | tc_3xtf32 | f64in_f32io | tc_3xf16 (gemm-type tasks)
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
+
+
+def bench_config(vs, **over):
+    """vs_config of the timed launch configuration (RT_DEFAULTS), keyword overrides on top."""
+    d = RT_DEFAULTS
+    kw = dict(lam=d["lam"], slots_per_gpu=d["slots"], priority=d["priority"], queue_depth=d["qdepth"],
+              group_tasks=d["group"], mode=1 if d["mode"] == "ready" else 0, group_hold=d["hold"],
+              group_wait_us=d["group_us"])
+    kw.update(over)
+    return vs.vs_config_default(**kw)
 
 
 def peaks():
@@ -137,7 +148,7 @@ class Workload:
         self.ids.extend(ids.values())
         return T, [ids[t] for t in tiles]
 
-    def reset(self):
+    def reset(self, sync=True):
         """Restore this rank's inputs (C = 0, A_chol = pristine) and declare EVERY datum
         modified (vs_data_invalidate), as if a new batch of inputs had been written: no
         replica, cached remote tile or derived operand form (tc_3xf16 split halves) of the
@@ -148,7 +159,7 @@ class Workload:
             self.C.zero_()
         if self.with_ch:
             self.S.copy_(self.S0)
-        if not self.host:
+        if not self.host and sync:
             self.torch.cuda.current_stream().synchronize()
         for d in self.ids:
             self.rt.vs_data_invalidate(d)
@@ -162,10 +173,14 @@ class Workload:
             rt.vs_app_cholesky(self.types, self.ch_nt, self.iS)
 
     def step(self, barrier=None):
-        self.reset()
+        # the restores run on the GPU while the host builds the step's task graph (vs_submit
+        # only records tasks and dependences; nothing is issued before vs_wait_all)
+        self.reset(sync=False)
+        self.submit()
+        if not self.host:
+            self.torch.cuda.current_stream().synchronize()
         if barrier:
             barrier()      # owners' resets done before any rank reads their tiles
-        self.submit()
         self.rt.vs_wait_all()
 
 
@@ -351,6 +366,10 @@ def main():
                     help="decide when predecessors completed (ready) or on the virtual clock (runahead)")
     ap.add_argument("--group", type=int, default=int(os.environ.get("VS_GROUP", RT_DEFAULTS["group"])),
                     help="tasks per grouped launch (vs_config.group_tasks)")
+    ap.add_argument("--hold", type=int, default=int(os.environ.get("VS_GROUP_HOLD", RT_DEFAULTS["hold"])),
+                    help="vs_config.group_hold: idle flush spares groups whose stream still runs a kernel")
+    ap.add_argument("--group-us", type=int, default=int(os.environ.get("VS_GROUP_US", RT_DEFAULTS["group_us"])),
+                    help="vs_config.group_wait_us")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--small", action="store_true", help="cfg1/cfg2-sized smoke of the bench itself")
@@ -393,7 +412,8 @@ def main():
     look = int(os.environ.get("VS_LOOKAHEAD", "0"))
     mode = 1 if args.mode == "ready" else 0          # VS_MODE_READY / VS_MODE_RUNAHEAD
     cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0,
-                               priority=prio, lookahead=look, queue_depth=qdepth, group_tasks=args.group, mode=mode)
+                               priority=prio, lookahead=look, queue_depth=qdepth, group_tasks=args.group, mode=mode,
+                               group_hold=args.hold, group_wait_us=args.group_us)
     rt = vs.Runtime(cfg)
     if world > 1:
         shm = gather("/vsched_%d_%d" % (os.getpid(), int(time.time())) if rank == 0 else None)[0]
@@ -463,7 +483,8 @@ def main():
     e2e = None
     if not args.no_e2e and world == 1:
         rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look,
-                                              queue_depth=qdepth, group_tasks=args.group, mode=mode))
+                                              queue_depth=qdepth, group_tasks=args.group, mode=mode,
+                                              group_hold=args.hold, group_wait_us=args.group_us))
         wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, with_mm=with_mm, with_ch=with_ch)
         wl2.step()     # warm-up incl. learning
         tsum, h2d, d2h = 0.0, 0, 0
@@ -517,6 +538,7 @@ def main():
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
             "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
             "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "group_tasks": args.group,
+                                "group_hold": args.hold, "group_wait_us": args.group_us,
                                 "mode": args.mode, "cuda_device_max_connections": os.environ.get("CUDA_DEVICE_MAX_CONNECTIONS")},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,

@@ -41,7 +41,7 @@ class vs_config(Structure):
                 ("lambda_", c_int), ("policy", c_int), ("fixed_version", c_int), ("learning", c_int),
                 ("mode", c_int), ("replay", c_int), ("flush", c_int), ("lookahead", c_int), ("priority", c_int),
                 ("group_ratio_permille", c_int), ("ewma_weight", c_int), ("locality_gbps", c_int),
-                ("queue_depth", c_int), ("group_tasks", c_int), ("group_wait_us", c_int)]
+                ("queue_depth", c_int), ("group_tasks", c_int), ("group_wait_us", c_int), ("group_hold", c_int)]
 
 
 class vs_stats_t(Structure):

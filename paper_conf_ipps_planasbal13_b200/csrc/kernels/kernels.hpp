@@ -25,7 +25,13 @@ struct TaskCtx {
     unsigned long long *host = nullptr;   // host-mapped {~start, end, kernels done, exec time}
     unsigned int ncta = 0;   // CTAs of the task in the launch (0: the whole grid)
     unsigned int nsm = 0;    // SMs of the device (CTAs that can run at once, 1 per SM)
+    // completion ring (host-mapped): the last CTA of every kernel of the task appends `tag`
+    // at ring[atomicAdd(ring_ctr) % kRingCap], so the host reads completions in O(completed)
+    unsigned long long *ring_ctr = nullptr;   // device counter of appended entries
+    unsigned long long *ring = nullptr;       // host-mapped entries (0 = empty)
+    unsigned long long tag = 0;               // task id + 1
 };
+constexpr unsigned long long kRingCap = 1ull << 16;
 
 // Task types / versions use the VS_T_* / VS_V_* numbering of vsched.h.
 // Returns 0 on success, -1 for an unsupported (type, version, b).

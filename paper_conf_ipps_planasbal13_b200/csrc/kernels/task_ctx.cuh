@@ -71,6 +71,12 @@ __device__ __forceinline__ void ctx_end(const TaskCtx &c)
                 // with the number of kernels the version launched) instead of querying events
                 __threadfence_system();
                 h[2] = h[2] + 1;
+                if (c.ring) {   // the record above is visible before the ring entry
+                    __threadfence_system();
+                    const unsigned long long pos = atomicAdd(c.ring_ctr, 1ull);
+                    volatile unsigned long long *r = c.ring;
+                    r[pos & (kRingCap - 1)] = c.tag;
+                }
             }
             atomicExch(&c.slot[2], 0ull);   // re-arm for the task's next kernel
         }

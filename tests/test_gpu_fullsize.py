@@ -1,7 +1,8 @@
 """Parity at BASELINE.json's full sizes, in the launch configuration bench.py times
-(cfg3 matmul N=16384 b=1024 + cfg4 Cholesky N=32768 b=1024, bench.RT_DEFAULTS: lambda 3,
-6 slots, bottom-level priority, queue depth 2; all f32 versions, run-ahead): sampled outputs the oracle computes one by one, plus properties that
-hold at any size."""
+(cfg3 matmul N=16384 b=1024 + cfg4 Cholesky N=32768 b=1024, bench.bench_config() = RT_DEFAULTS:
+lambda 3, 12 slots, ready mode, bottom-level priority, queue depth 2, grouped launches with
+group_hold; all f32 versions): sampled outputs the oracle computes one by one, plus properties
+that hold at any size."""
 import numpy as np
 import pytest
 
@@ -16,9 +17,7 @@ def test_fullsize_bench_configuration(gpu):
     import torch
 
     import bench
-    d = bench.RT_DEFAULTS
-    rt = vs.Runtime(vs.vs_config_default(lam=d["lam"], slots_per_gpu=d["slots"], priority=d["priority"],
-                                         queue_depth=d["qdepth"]))
+    rt = vs.Runtime(bench.bench_config(vs))
     wl = bench.Workload(rt)
     wl.step()          # learning happens here (cold)
     wl.step()          # warm step, as timed by bench.py
