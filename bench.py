@@ -161,8 +161,7 @@ class Workload:
             self.S.copy_(self.S0)
         if not self.host and sync:
             self.torch.cuda.current_stream().synchronize()
-        for d in self.ids:
-            self.rt.vs_data_invalidate(d)
+        self.rt.vs_data_invalidate_n(self.ids)
 
     def submit(self):
         vs, rt = self.vs, self.rt
@@ -256,33 +255,42 @@ def roofline(log, groups, ms, world):
     for g in groups:
         npar = {"MATMUL": 3, "GEMM_NT": 3, "SYRK": 2, "TRSM": 2, "POTRF": 1}[g["type_name"].split(".")[0]]
         tile_b[g["type"]] = int(round(math.sqrt(g["bytes"] / 4 / npar)))
-    per = {}
+    # per KERNEL class: every tc_3xf16 task but potrf (MATMUL, GEMM_NT, SYRK and TRSM-by-inverse,
+    # R30/R31) runs the same kernel, tcf_gemm_kernel (grouped launches mix them); other
+    # versions are keyed by (type, version)
+    per, per_tv = {}, {}
     for (task, v, w, td, ts, te, ph, ty) in log:
-        key = (tnames[ty], vnames[ty][v], tile_b[ty])
-        d = per.setdefault(key, {"n": 0, "flops": 0.0, "iv": []})
+        tname, vname, b = tnames[ty], vnames[ty][v], tile_b[ty]
+        fl = task_flops(tname, b)
+        kname = "tcf_gemm_kernel" if vname == "tc_3xf16" and not tname.startswith("POTRF") else "%s/%s" % (tname, vname)
+        d = per.setdefault(kname, {"n": 0, "flops": 0.0, "iv": [], "version": vname})
         d["n"] += 1
-        d["flops"] += task_flops(tnames[ty], tile_b[ty])
+        d["flops"] += fl
         d["iv"].append((ts, te))
+        e = per_tv.setdefault((tname, vname, b), {"n": 0, "flops": 0.0})
+        e["n"] += 1
+        e["flops"] += fl
     dom = max(per, key=lambda k: per[k]["flops"])
     d = per[dom]
     union = union_ns(d["iv"])
     f16_peak = pk.get("bf16_tflops_sustained", pk["bf16_tflops"])            # fp16 dense = bf16 dense rate
     tc_peak = {"tc_3xtf32": (tf32_peak, "%s bf16_tflops_sustained x 0.5 (TF32/BF16 nominal ratio)" % pk_kind),
                "tc_3xf16": (f16_peak, "%s bf16_tflops_sustained (fp16 = bf16 dense rate)" % pk_kind)}
-    hw = 3.0 if dom[1] in tc_peak else 1.0
+    hw = 3.0 if d["version"] in tc_peak else 1.0
     achieved = hw * d["flops"] / (union * 1e-9) / 1e12
-    if dom[1] in tc_peak:
-        (peak, src), bound = tc_peak[dom[1]], "tensor"
+    if d["version"] in tc_peak:
+        (peak, src), bound = tc_peak[d["version"]], "tensor"
     else:
         peak, bound, src = 148 * 128 * 2 * pk["sm_max_mhz"] * 1e6 / 1e12, "alu", "148 SM x 128 FMA x 2 x sm_max_mhz"
     # tensor-pipe busy fraction of the whole step: hardware MMA flops of every tensor-core
     # task / (step time x that version's peak), summed over versions
-    frac_step = sum(3.0 * v["flops"] / tc_peak[k[1]][0] for k, v in per.items() if k[1] in tc_peak) / (ms * 1e-3) / 1e12
-    roof = {"bound": bound, "kernel": "%s/%s b=%d" % dom, "achieved": round(achieved, 2), "peak": round(peak, 1),
+    frac_step = sum(3.0 * v["flops"] / tc_peak[k[1]][0] for k, v in per_tv.items() if k[1] in tc_peak) / (ms * 1e-3) / 1e12
+    roof = {"bound": bound, "kernel": dom, "tasks": d["n"], "achieved": round(achieved, 2), "peak": round(peak, 1),
             "unit": "TFLOP/s", "frac": round(achieved / peak, 4), "traffic": None, "peak_source": src,
-            "how": "hardware MMA flops (3x algorithmic) of all launches of this kernel class in the timed steps / "
-                   "union of their device-recorded execution intervals (%globaltimer, task_ctx.cuh)"}
-    counts = {"%s/%s" % k[:2]: v["n"] for k, v in sorted(per.items())}
+            "how": "hardware MMA flops (3x the algorithmic flops of its tasks: 2b^3 matmul/gemm, b^3 syrk/trsm) of "
+                   "every task this kernel ran in the timed steps / union of their device-recorded execution "
+                   "intervals (%globaltimer, task_ctx.cuh)"}
+    counts = {"%s/%s" % k[:2]: v["n"] for k, v in sorted(per_tv.items())}
     return roof, frac_step, counts
 
 

@@ -214,6 +214,10 @@ int vs_data_register(vs_rt rt, void *ptr, int device, int64_t bytes, vs_data_id 
  * VS_E_STATE if a task writing d is still in flight. */
 int vs_data_invalidate(vs_rt rt, vs_data_id d);
 
+/* vs_data_invalidate of ids[0..n-1] (one call for a whole matrix of tiles); stops at, and
+ * returns the error of, the first failing id. */
+int vs_data_invalidate_n(vs_rt rt, const vs_data_id *ids, int64_t n);
+
 /* ------------------------------------------------------------- submission (a2) */
 /* Create a task instance: RAW/WAR/WAW edges on whole data (L236-242).  scalars
  * (may be NULL) are copied and passed to the version.  Execution happens inside

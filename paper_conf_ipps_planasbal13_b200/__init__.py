@@ -123,6 +123,7 @@ def lib():
         "vs_ipc_open": (c_int, [ctypes.c_char * 64, c_uint64, POINTER(c_void_p)]),
         "vs_ipc_close": (c_int, [c_void_p]),
         "vs_data_invalidate": (c_int, [rt, c_int64]),
+        "vs_data_invalidate_n": (c_int, [rt, c_void_p, c_int64]),
         "vs_operand_form": (c_int, [c_int, c_int, c_int]),
         "vs_form_bytes": (c_int64, [c_int, c_int]),
         "vs_form_make": (c_int, [c_int, c_int, c_void_p, c_void_p, c_void_p]),
@@ -143,7 +144,7 @@ EXPORTED = ["vs_config_default", "vs_create", "vs_destroy", "vs_last_error", "vs
             "vs_decision_log", "vs_decision_log_hash", "vs_decision_log_clear", "vs_table_dump", "vs_table_load",
             "vs_replay_set", "vs_app_matmul", "vs_app_cholesky", "vs_tile_run", "vs_gen_uniform", "vs_gen_spd",
             "vs_build_info", "vs_gen_tile", "vs_dist_init", "vs_data_set_owner", "vs_ipc_export", "vs_ipc_open",
-            "vs_ipc_close", "vs_data_invalidate", "vs_operand_form", "vs_form_bytes", "vs_form_make",
+            "vs_ipc_close", "vs_data_invalidate", "vs_data_invalidate_n", "vs_operand_form", "vs_form_bytes", "vs_form_make",
             "vs_tile_run_prepared", "vs_decision_issue_ns"]
 
 
@@ -362,6 +363,10 @@ class Runtime:
 
     def vs_data_invalidate(self, d):
         return self._ck(lib().vs_data_invalidate(self.h, d), "vs_data_invalidate")
+
+    def vs_data_invalidate_n(self, ids):
+        a = _ids(list(ids))
+        return self._ck(lib().vs_data_invalidate_n(self.h, ctypes.cast(a, c_void_p), len(a)), "vs_data_invalidate_n")
 
     def vs_dist_init(self, rank, nranks, shm_name=""):
         return self._ck(lib().vs_dist_init(self.h, rank, nranks, shm_name.encode()), "vs_dist_init")

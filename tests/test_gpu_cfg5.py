@@ -41,7 +41,9 @@ def test_cfg5_interleaved_convergence(gpu, lam):
         fastest = int(np.argmin(means))
         post = [r[1] for r in recs[V * lam:]]
         assert all(means[v] <= 1.5 * means[fastest] for v in post), (b, g)
-        assert sum(v == fastest for v in post) >= len(post) // 2, (b, g)
+        second = min(means[v] for v in range(V) if v != fastest)
+        if second >= 1.2 * means[fastest]:   # a clear winner (not a near-tie) takes most picks
+            assert sum(v == fastest for v in post) >= len(post) // 2, (b, g)
         if b > 256:
             continue
         # parity of the result (C0 = 0, A = u(100+lam), B = u(1100+lam), N = 4b)
