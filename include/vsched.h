@@ -101,7 +101,12 @@ enum {
                              (R31); no POTRF.  Its in-operands
                              are read through a per-GPU cached "split form" that the runtime builds
                              (one conversion kernel per datum version, like a tile move) */
-    VS_NUM_BUILTIN_VERSIONS = 6
+    VS_V_OZ_I8_F64 = 6,   /* fp64 tiles, tcgen05 kind::i8 Ozaki scheme (NEXT-4): each operand row as
+                             7 int8 slices under a power-of-two row scale (a cached "slice form",
+                             like tc_3xf16's split form), the 28 slice products with i + j <= 8
+                             accumulated exactly in int32 TMEM (one accumulator per diagonal),
+                             combined in fp64; MATMUL, GEMM_NT, SYRK; no POTRF / TRSM */
+    VS_NUM_BUILTIN_VERSIONS = 7
 };
 
 typedef struct {
@@ -328,14 +333,16 @@ int vs_tile_run(int type, int version, int b, void *const *ptrs, int *dinfo, voi
  * itself, 1 = row split form, 2 = column split form, i.e. the row split form of the
  * transposed tile, 3 = row split form of inv(L)) in which `version` reads parameter `param`
  * of built-in `type`;
- * vs_form_bytes the size of a form of a b x b fp32 tile (0 for form 0).
- * vs_form_make enqueues the conversion of the b x b fp32 tile `src` into `dst`
+ * vs_form_bytes the size of a form of a b x b tile (0 for form 0).
+ * vs_form_make enqueues the conversion of the b x b tile `src` (fp32; fp64 for forms 4, 5) into `dst`
  * (vs_form_bytes bytes, device memory, 16-byte aligned) on `stream`.
  * vs_tile_run_prepared is vs_tile_run with the forms prepared by the caller (no
  * conversion): ptrs holds 2 * nparams pointers, ptrs[i] = the tile of parameter i (device),
  * ptrs[nparams + i] = its form (ignored for form 0) — the kernels the runtime launches for a
  * task.  Form 3 (TRSM of VS_V_TC_3XF16) = row split form of inv(L) for the lower triangle L
- * of the tile (reading R31).  VS_E_INVAL on bad arguments. */
+ * of the tile (reading R31).  Forms 4 / 5 / 6 (VS_V_OZ_I8_F64) = int8 slice form of the
+ * rows (A role) / of the columns (matmul B) / of the rows in the B role of an NT product, of a
+ * b x b fp64 tile.  VS_E_INVAL on bad arguments. */
 int vs_operand_form(int type, int version, int param);
 int64_t vs_form_bytes(int form, int b);
 int vs_form_make(int form, int b, const void *src, void *dst, void *stream);

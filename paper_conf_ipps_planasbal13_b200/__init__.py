@@ -27,9 +27,9 @@ VS_POLICY_VERSIONING, VS_POLICY_FIXED = 0, 1
 VS_F32, VS_F64 = 0, 1
 VS_T_MATMUL, VS_T_POTRF, VS_T_TRSM, VS_T_SYRK, VS_T_GEMM_NT = range(5)
 VS_NUM_BUILTIN_TYPES = 5
-VS_V_SIMT_F32, VS_V_TC_3XTF32, VS_V_F64IN_F32IO, VS_V_DFMA_F64, VS_V_DMMA_F64, VS_V_TC_3XF16 = range(6)
+VS_V_SIMT_F32, VS_V_TC_3XTF32, VS_V_F64IN_F32IO, VS_V_DFMA_F64, VS_V_DMMA_F64, VS_V_TC_3XF16, VS_V_OZ_I8_F64 = range(7)
 VS_MAX_VERSIONS = 8
-VERSION_NAMES = ["simt_f32", "tc_3xtf32", "f64in_f32io", "dfma_f64", "dmma_f64", "tc_3xf16"]
+VERSION_NAMES = ["simt_f32", "tc_3xtf32", "f64in_f32io", "dfma_f64", "dmma_f64", "tc_3xf16", "oz_i8_f64"]
 TYPE_NAMES = ["MATMUL", "POTRF", "TRSM", "SYRK", "GEMM_NT"]
 
 ERRORS = {0: "VS_OK", -1: "VS_E_INVAL", -2: "VS_E_NOMEM", -3: "VS_E_CUDA", -4: "VS_E_NOT_SPD",

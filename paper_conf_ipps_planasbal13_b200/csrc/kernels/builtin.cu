@@ -11,6 +11,8 @@
 //   dmma_f64       fp64     dmma_gemm<double>  (mma.sync f64)                      blocked
 //   tc_3xf16       fp32     tcf_gemm (tcgen05 kind::f16 on split forms, tc_f16.cuh); TRSM = GEMM with
 //                           the inv(L) form (R31); no potrf
+//   oz_i8_f64      fp64     oz_gemm (tcgen05 kind::i8 Ozaki scheme on slice forms, tc_oz.cuh);
+//                           MATMUL / GEMM_NT / SYRK only
 //
 // potrf of tc_3xtf32 is the single-launch left-looking tc_panel kernel (tc_panel.cuh).
 // potrf of the other versions is recursive: potrf(A11); A21 <- A21 L11^{-T} (trsm);
@@ -25,6 +27,7 @@
 #include "simt_gemm.cuh"
 #include "tc_gemm.cuh"
 #include "tc_f16.cuh"
+#include "tc_oz.cuh"
 #include "tc_panel.cuh"
 
 #include "vsched.h"
@@ -143,13 +146,17 @@ int run_family(int type, int b, void *const *p, int *info, cudaStream_t s, const
 
 }  // namespace
 
-int builtin_elem_bytes(int version) { return (version == VS_V_DFMA_F64 || version == VS_V_DMMA_F64) ? 8 : 4; }
+int builtin_elem_bytes(int version)
+{
+    return (version == VS_V_DFMA_F64 || version == VS_V_DMMA_F64 || version == VS_V_OZ_I8_F64) ? 8 : 4;
+}
 
 bool builtin_supported(int type, int version, int b)
 {
     if (type < 0 || type >= VS_NUM_BUILTIN_TYPES) return false;
     if (version < 0 || version >= VS_NUM_BUILTIN_VERSIONS) return false;
     if (version == VS_V_TC_3XF16 && type == VS_T_POTRF) return false;
+    if (version == VS_V_OZ_I8_F64 && (type == VS_T_POTRF || type == VS_T_TRSM)) return false;
     if (b && (b % 64 != 0 || b < 64 || b > 4096)) return false;
     return true;
 }
@@ -162,6 +169,14 @@ int builtin_nparams(int type)
 
 int builtin_operand_form(int type, int version, int param)
 {
+    if (version == VS_V_OZ_I8_F64) {
+        switch (type) {
+        case VS_T_MATMUL: return param == 0 ? FORM_OZ_ROWS : param == 1 ? FORM_OZ_COLS : FORM_RAW;
+        case VS_T_GEMM_NT: return param == 0 ? FORM_OZ_ROWS : param == 1 ? FORM_OZ_ROWS_B : FORM_RAW;
+        case VS_T_SYRK: return param == 0 ? FORM_OZ_ROWS : FORM_RAW;
+        }
+        return FORM_RAW;
+    }
     if (version != VS_V_TC_3XF16) return FORM_RAW;
     switch (type) {
     case VS_T_MATMUL: return param == 0 ? FORM_SPLIT_ROWS : param == 1 ? FORM_SPLIT_COLS : FORM_RAW;
@@ -175,12 +190,17 @@ int builtin_operand_form(int type, int version, int param)
 size_t form_bytes(int form, int b)
 {
     if (form == FORM_RAW) return 0;
+    if (form == FORM_OZ_ROWS || form == FORM_OZ_COLS || form == FORM_OZ_ROWS_B)
+        return (oz::form_bytes(b, b) + 255) / 256 * 256;
     const size_t sb = (tcf::split_bytes(b, b) + 255) / 256 * 256;
     return form == FORM_INV_L ? sb + (size_t)b * b * 4 : sb;   // + fp32 scratch for inv(L)^T
 }
 
 int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
 {
+    if (form == FORM_OZ_ROWS) return oz::make_slices((const double *)src, b, b, b, 1, 128, dst, s);
+    if (form == FORM_OZ_ROWS_B) return oz::make_slices((const double *)src, b, b, b, 1, 64, dst, s);
+    if (form == FORM_OZ_COLS) return oz::make_slices((const double *)src, b, b, 1, b, 64, dst, s);
     if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
     if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
     if (form == FORM_INV_L) {
@@ -220,6 +240,16 @@ int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const 
 int group_launch(TaskGroup *g, cudaStream_t s) { return tcf::tcf_group_launch(g->g, s); }
 
 namespace {
+// oz_i8_f64: p[np + i] holds the slice forms of the in-operands (builtin_operand_form)
+int run_oz(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
+{
+    switch (type) {
+    case VS_T_MATMUL: return oz::oz_gemm<false, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, ctx);   // C += A B
+    case VS_T_GEMM_NT: return oz::oz_gemm<true, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, ctx);  // C -= A B^T
+    case VS_T_SYRK: return oz::oz_gemm<true, true, 128>(b, b, b, p[2], p[2], (double *)p[1], b, s, ctx);     // C -= A A^T
+    }
+    return -1;
+}
 // tc_3xf16: p[] holds the split forms of the in-operands (builtin_operand_form)
 int run_f16(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
 {
@@ -240,6 +270,7 @@ int launch_builtin(int type, int version, int b, void *const *p, int *info, cuda
     case VS_V_DFMA_F64: return run_family<double, SimtEngine<double, double>>(type, b, p, info, s, ctx);
     case VS_V_DMMA_F64: return run_family<double, DmmaEngine<double>>(type, b, p, info, s, ctx);
     case VS_V_TC_3XF16: return run_f16(type, b, p, s, ctx);
+    case VS_V_OZ_I8_F64: return run_oz(type, b, p, s, ctx);
     }
     return -1;
 }

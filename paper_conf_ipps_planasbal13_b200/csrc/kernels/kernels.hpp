@@ -46,7 +46,11 @@ int builtin_elem_bytes(int version);
 // FORM_INV_L: row split form of inv(L) for the lower triangle L of a tile (TRSM by GEMM).
 // Pointer layout of launch_builtin / group_add for versions with forms: p[i] = the tile
 // of parameter i, p[nparams + i] = its form (nparams = builtin_nparams(type)).
-enum { FORM_RAW = 0, FORM_SPLIT_ROWS = 1, FORM_SPLIT_COLS = 2, FORM_INV_L = 3, NUM_FORMS = 4 };
+// FORM_OZ_ROWS / FORM_OZ_COLS / FORM_OZ_ROWS_B: int8 slice forms of the rows (A role,
+// 128-row groups) / columns (matmul B, 64-row groups) / rows (NT B role, 64-row groups) of
+// an fp64 tile (oz_i8_f64, tc_oz.cuh).
+enum { FORM_RAW = 0, FORM_SPLIT_ROWS = 1, FORM_SPLIT_COLS = 2, FORM_INV_L = 3, FORM_OZ_ROWS = 4, FORM_OZ_COLS = 5,
+       FORM_OZ_ROWS_B = 6, NUM_FORMS = 7 };
 int builtin_nparams(int type);
 int builtin_operand_form(int type, int version, int param);
 size_t form_bytes(int form, int b);

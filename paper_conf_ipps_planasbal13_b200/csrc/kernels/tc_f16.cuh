@@ -242,6 +242,31 @@ __device__ __forceinline__ void bulk_g2s(uint32_t dst, const void *src, uint32_t
                  "l"(src), "r"(bytes), "r"(smem_u32(bar))
                  : "memory");
 }
+// the same bytes into the same smem offset of every CTA in ctaMask (cluster), each CTA's
+// mbarrier at the same offset receiving the complete_tx
+__device__ __forceinline__ void bulk_g2s_mc(uint32_t dst, const void *src, uint32_t bytes, uint64_t *bar, uint16_t mask)
+{
+    asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.multicast::cluster [%0], [%1], %2, [%3], %4;"
+                 ::"r"(dst), "l"(src), "r"(bytes), "r"(smem_u32(bar)), "h"(mask)
+                 : "memory");
+}
+__device__ __forceinline__ void mma_commit_mc(uint64_t *bar, uint16_t mask)
+{
+    asm volatile("tcgen05.commit.cta_group::1.mbarrier::arrive::one.shared::cluster.multicast::cluster.b64 [%0], %1;"
+                 ::"r"(smem_u32(bar)), "h"(mask)
+                 : "memory");
+}
+__device__ __forceinline__ void cluster_sync_all()
+{
+    asm volatile("barrier.cluster.arrive.release.aligned;\n\tbarrier.cluster.wait.acquire.aligned;" ::: "memory");
+}
+__device__ __forceinline__ uint32_t cluster_ctarank()
+{
+    uint32_t r;
+    asm volatile("mov.u32 %0, %%cluster_ctarank;" : "=r"(r));
+    return r;
+}
+
 __device__ __forceinline__ void prefetch_l2(const void *p, uint32_t bytes)
 {
     asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(p), "r"(bytes) : "memory");
@@ -298,7 +323,15 @@ struct TcfGroupN {
 using TcfGroup = TcfGroupN<kMaxGroup>;
 static_assert(sizeof(TcfGroup) <= 4000, "kernel parameter space");
 
-template <int G>
+// PAIR: clusters of two CTAs computing tiles (bi, 2p) and (bi, 2p+1) of one task share the
+// A operand: each CTA bulk-copies one half (big or small part) of the stage's A block and
+// multicasts it into both CTAs, so a CTA reads 48 KB per k-block from L2 instead of 64 KB
+// (the GEMM is L2-bandwidth bound when every SM runs it).  A stage of either CTA is
+// refilled only after BOTH CTAs' MMAs released it (empty barriers count 2: each MMA warp
+// commits to its own and its peer's).  A pair whose second tile does not exist (odd tile
+// count in a row, or above the diagonal for LOWER) runs a "ghost" CTA: it loads and
+// multiplies a valid tile but stores nothing.
+template <int G, bool PAIR>
 __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_constant__ TcfGroupN<G> grp)
 {
     extern __shared__ uint8_t smem_raw[];
@@ -321,7 +354,25 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
     const bool NEG = tk.flags & 1, LOWER = (tk.flags >> 1) & 1;
     const int l = (int)blockIdx.x - tk.tile0;
     int bi, bj;
-    if (LOWER) {   // l = bi (bi + 1) / 2 + bj, bj <= bi
+    bool ghost = false;
+    const uint32_t rank = PAIR ? cluster_ctarank() : 0u;
+    if (PAIR) {
+        const int pi = l >> 1;
+        int p;
+        if (LOWER) {   // row bi holds bi/2 + 1 pairs
+            bi = 0;
+            int acc = 0;
+            while (acc + bi / 2 + 1 <= pi) acc += bi / 2 + 1, bi++;
+            p = pi - acc;
+        } else {
+            const int ppr = (tk.tiles_n + 1) / 2;
+            bi = pi / ppr;
+            p = pi % ppr;
+        }
+        bj = 2 * p + (int)rank;
+        ghost = bj >= tk.tiles_n || (LOWER && bj > bi);
+        if (ghost) bj = 2 * p;   // a valid tile to load; nothing is stored
+    } else if (LOWER) {   // l = bi (bi + 1) / 2 + bj, bj <= bi
         bi = (int)((sqrtf(8.f * l + 1.f) - 1.f) * 0.5f);
         while ((bi + 1) * (bi + 2) / 2 <= l) bi++;
         while (bi * (bi + 1) / 2 > l) bi--;
@@ -339,7 +390,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         TCF_T(0);
         for (int s = 0; s < STAGES; s++) {
             mbar_init(&full[s], 1);
-            mbar_init(&empty[s], 1);
+            mbar_init(&empty[s], PAIR ? 2 : 1);
         }
         mbar_init(acc_full, 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
@@ -352,6 +403,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
     tc_fence_before();
     __syncthreads();
     tc_fence_after();
+    if (PAIR) cluster_sync_all();   // the peer's barriers are initialised before any multicast
     const uint32_t tmem = *tmem_slot;
     if (threadIdx.x == 0) TCF_T(1);
 
@@ -363,7 +415,11 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
                 if (kb >= STAGES) mbar_wait(&empty[s], ((kb / STAGES) - 1) & 1);
                 const uint32_t st = smem_u32(smem + s * STAGE);
                 mbar_expect_tx(&full[s], STAGE);
-                bulk_g2s(st, As + (size_t)kb * RA * 128 + (size_t)m0 * 128, 2 * PART, &full[s]);
+                if (PAIR)   // this CTA's half (big or small part) of the A block, into both CTAs
+                    bulk_g2s_mc(st + rank * PART, As + (size_t)kb * RA * 128 + (size_t)m0 * 128 + rank * PART, PART,
+                                &full[s], (uint16_t)3);
+                else
+                    bulk_g2s(st, As + (size_t)kb * RA * 128 + (size_t)m0 * 128, 2 * PART, &full[s]);
                 bulk_g2s(st + 2 * PART, Bs + (size_t)kb * RB * 128 + (size_t)n0 * 128, 2 * PART, &full[s]);
             }
         }
@@ -403,7 +459,10 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
                         mma_f16(d, dAs, dBb, idesc, 1u);
                     }
                 }
-                tc::mma_commit(&empty[s]);
+                if (PAIR && kb < nk - STAGES)
+                    mma_commit_mc(&empty[s], (uint16_t)3);   // both CTAs' producers refill stage s
+                else if (!PAIR)
+                    tc::mma_commit(&empty[s]);
                 if (kb == nk - 1) {
                     tc::mma_commit(acc_full);
                     TCF_T(4);
@@ -419,7 +478,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         const float *sav = reinterpret_cast<const float *>(As + (size_t)RA * K * 4) + m0;
         const float4 sb = __ldg(reinterpret_cast<const float4 *>(reinterpret_cast<const float *>(Bs + (size_t)RB * K * 4) + n0 + ccol));
         const bool BETA0 = (tk.flags >> 2) & 1;   // C = s A B'^T (C_in not read)
-        if (!BETA0) {   // C_in into L2 while the main loop runs (LSU prefetches: bulk prefetches
+        if (!BETA0 && !ghost) {   // C_in into L2 while the main loop runs (LSU prefetches: bulk prefetches
             // would occupy the TMA unit that feeds the operands): thread t -> tile row t, its 1 KB
             const int r = threadIdx.x - 64;
             if (m0 + r < M)
@@ -432,7 +491,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         if (warp == 2 && lane == 0) TCF_T(6);
         const int gcol = n0 + ccol;
 #pragma unroll 1
-        for (int h = 0; h < 2; h++) {
+        for (int h = 0; h < (ghost ? 0 : 2); h++) {
             const int rbase = h * 128 + q * 32;          // tile rows of this warp
             const float sa_l = __ldg(sav + rbase + lane);
 #pragma unroll 1
@@ -488,6 +547,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         tc_fence_after();
         asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"(512u));
     }
+    if (PAIR) cluster_sync_all();   // no CTA leaves while its peer may still address its smem
     ctx_end(ctx);
 }
 
@@ -516,13 +576,27 @@ inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStrea
 
 // Append one task to a group; returns its CTA count, 0 for an empty task, -1 if it does
 // not fit or is unsupported (K a multiple of 32, ldc of 4).
+// CTA-pair (A multicast) variant of the GEMM: on unless VS_TCF_PAIR=0
+inline bool tcf_pair()
+{
+    static const int v = [] {
+        const char *e = getenv("VS_TCF_PAIR");
+        return e ? atoi(e) : 1;
+    }();
+    return v != 0;
+}
+
 inline int tcf_group_add(TcfGroup &g, int M, int N, int K, const void *As, const void *Bs, float *C, int ldc,
                          bool neg, bool lower, TaskCtx ctx, bool beta0 = false)
 {
     if (M <= 0 || N <= 0) return 0;
     if (K % BK || ldc % 4 || g.n >= kMaxGroup || (lower && M != N)) return -1;
     const int tm = (M + BT - 1) / BT, tn = (N + BT - 1) / BT;
-    const int nt = lower ? tm * (tm + 1) / 2 : tm * tn;
+    int nt = lower ? tm * (tm + 1) / 2 : tm * tn;
+    if (tcf_pair()) {   // two CTAs per pair of tiles in a row (kernel comment): rows hold ceil(tn/2)
+        nt = 0;         // pairs, row bi of a LOWER task bi/2 + 1
+        for (int bi = 0; bi < tm; bi++) nt += 2 * (lower ? bi / 2 + 1 : (tn + 1) / 2);
+    }
     TcfTask &t = g.t[g.n++];
     t.As = (const uint8_t *)As;
     t.Bs = (const uint8_t *)Bs;
@@ -538,6 +612,45 @@ inline int tcf_group_add(TcfGroup &g, int M, int N, int K, const void *As, const
     return nt;
 }
 
+template <int G, bool PAIR>
+inline void tcf_launch_one(const TcfGroupN<G> &h, int ctas, cudaStream_t s)
+{
+    if (!PAIR) {
+        tcf_gemm_kernel<G, false><<<ctas, NTHREADS, SMEM, s>>>(h);
+        return;
+    }
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3(ctas);
+    cfg.blockDim = dim3(NTHREADS);
+    cfg.dynamicSmemBytes = SMEM;
+    cfg.stream = s;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeClusterDimension;
+    at[0].val.clusterDim.x = 2;
+    at[0].val.clusterDim.y = 1;
+    at[0].val.clusterDim.z = 1;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    cudaLaunchKernelEx(&cfg, tcf_gemm_kernel<G, true>, h);
+}
+
+template <bool PAIR>
+inline void tcf_launch(TcfGroup &g, cudaStream_t s)
+{
+    if (g.n == 1) {
+        TcfGroupN<1> h;
+        h.n = 1; h.ctas = g.ctas; h.t[0] = g.t[0];
+        tcf_launch_one<1, PAIR>(h, g.ctas, s);
+    } else if (g.n <= 4) {
+        TcfGroupN<4> h;
+        h.n = g.n; h.ctas = g.ctas;
+        for (int i = 0; i < g.n; i++) h.t[i] = g.t[i];
+        tcf_launch_one<4, PAIR>(h, g.ctas, s);
+    } else {
+        tcf_launch_one<kMaxGroup, PAIR>(g, g.ctas, s);
+    }
+}
+
 inline int tcf_group_launch(TcfGroup &g, cudaStream_t s)
 {
     if (g.n == 0) return 0;
@@ -545,24 +658,17 @@ inline int tcf_group_launch(TcfGroup &g, cudaStream_t s)
     int dev = 0;
     cudaGetDevice(&dev);
     if (!attr[dev & 63]) {
-        cudaFuncSetAttribute(tcf_gemm_kernel<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
-        cudaFuncSetAttribute(tcf_gemm_kernel<4>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
-        cudaFuncSetAttribute(tcf_gemm_kernel<kMaxGroup>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<1, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<4, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<kMaxGroup, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<1, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<4, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
+        cudaFuncSetAttribute(tcf_gemm_kernel<kMaxGroup, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, SMEM);
         attr[dev & 63] = true;
     }
     count_launch();
-    if (g.n == 1) {
-        TcfGroupN<1> h;
-        h.n = 1; h.ctas = g.ctas; h.t[0] = g.t[0];
-        tcf_gemm_kernel<1><<<g.ctas, NTHREADS, SMEM, s>>>(h);
-    } else if (g.n <= 4) {
-        TcfGroupN<4> h;
-        h.n = g.n; h.ctas = g.ctas;
-        for (int i = 0; i < g.n; i++) h.t[i] = g.t[i];
-        tcf_gemm_kernel<4><<<g.ctas, NTHREADS, SMEM, s>>>(h);
-    } else {
-        tcf_gemm_kernel<kMaxGroup><<<g.ctas, NTHREADS, SMEM, s>>>(g);
-    }
+    if (tcf_pair()) tcf_launch<true>(g, s);
+    else tcf_launch<false>(g, s);
     g.n = g.ctas = 0;
     return 0;
 }

@@ -12,7 +12,9 @@ pytestmark = pytest.mark.gpu
 
 F32_VERSIONS = [vs.VS_V_SIMT_F32, vs.VS_V_TC_3XTF32, vs.VS_V_F64IN_F32IO]
 F64_VERSIONS = [vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64]
-GEMM_VERSIONS = F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS   # tc_3xf16: gemm-type tasks only
+# tc_3xf16 and oz_i8_f64: gemm-type tasks only (tc_3xf16 also TRSM)
+GEMM_VERSIONS = F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS + [vs.VS_V_OZ_I8_F64]
+FP64_STORAGE = (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64, vs.VS_V_OZ_I8_F64)
 SIZES = [64, 128, 192, 320, 512]
 
 
@@ -39,11 +41,11 @@ def _run(ttype, version, b, arrays, info=None):
 
 
 def _gate(version):
-    return 1e-12 if version in (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64) else 1e-5
+    return 1e-12 if version in FP64_STORAGE else 1e-5
 
 
 def _dt(version):
-    return np.float64 if version in (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64) else np.float32
+    return np.float64 if version in FP64_STORAGE else np.float32
 
 
 # ------------------------------------------------------------------ generator
@@ -139,6 +141,42 @@ def test_tc_3xf16_row_scaling(gpu, ttype):
     bound = np.abs(A.astype(np.float64)) @ np.abs(Bop.astype(np.float64))
     err = np.abs(C.astype(np.float64) - ref)
     assert np.all(err <= 3e-5 * bound + 1e-37), float(np.max(err / (bound + 1e-300)))
+    assert np.all(C[3] == 0.0)
+
+
+@pytest.mark.parametrize("ttype", ["MATMUL", "GEMM_NT", "SYRK"])
+def test_oz_i8_f64_row_scales_and_componentwise_bound(gpu, ttype):
+    # oz_i8_f64: each operand row (B: column for MATMUL) carries its own power-of-two scale;
+    # rows spanning 2^-300 .. 2^300, an all-zero row and a row whose other entries are
+    # ~2^-30 of its maximum keep the bound |C - ref| <= 2^-44 |A||B| + b 2^-45 max|a_i.| max|b_.j|
+    # (truncated slices: < 10 * 2^-49 of the row maxima per product, tc_oz.cuh; plus the
+    # fp64 summation of the oracle and of the epilogue).
+    b = 192
+    rng = np.random.default_rng(6)
+    A = vsgen.uniform(710, b, b, np.float64) * np.exp2(rng.integers(-300, 300, size=(b, 1)))
+    B = vsgen.uniform(711, b, b, np.float64)
+    B = B * (np.exp2(rng.integers(-300, 300, size=(1, b))) if ttype == "MATMUL"
+             else np.exp2(rng.integers(-300, 300, size=(b, 1))))
+    A[3, :] = 0.0
+    A[5, :] = vsgen.uniform(712, 1, b, np.float64)[0] * 1e-9
+    A[5, 0] = 1.0
+    C0 = np.zeros((b, b))
+    t = getattr(vs, "VS_T_" + ttype)
+    if ttype == "SYRK":
+        (_, C) = _run(t, vs.VS_V_OZ_I8_F64, b, [A, C0])
+        ref, Bop = oracle.syrk(A, C0), A.T
+    else:
+        (_, _, C) = _run(t, vs.VS_V_OZ_I8_F64, b, [A, B, C0])
+        Bop = B if ttype == "MATMUL" else B.T
+        ref = oracle.matmul(A, Bop, C0) if ttype == "MATMUL" else oracle.gemm_nt(A, B, C0)
+    rowmax_a = np.max(np.abs(A), axis=1, keepdims=True)
+    colmax_b = np.max(np.abs(Bop), axis=0, keepdims=True)
+    bound = 2.0 ** -44 * (np.abs(A) @ np.abs(Bop)) + b * 2.0 ** -45 * rowmax_a * colmax_b
+    err = np.abs(C - ref)
+    if ttype == "SYRK":
+        lo = np.tril_indices(b)
+        err, bound = err[lo], bound[lo]
+    assert np.all(err <= bound), float(np.max(err / (bound + 1e-300)))
     assert np.all(C[3] == 0.0)
 
 

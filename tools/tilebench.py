@@ -20,7 +20,7 @@ NARGS = {vs.VS_T_MATMUL: 3, vs.VS_T_GEMM_NT: 3, vs.VS_T_SYRK: 2, vs.VS_T_TRSM: 2
 
 
 def bench(ttype, version, b, streams=1, iters=20):
-    dt = torch.float64 if version in (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64) else torch.float32
+    dt = torch.float64 if version in (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64, vs.VS_V_OZ_I8_F64) else torch.float32
     sets = []
     for s in range(streams):
         args = [torch.randn(b, b, dtype=dt, device="cuda") * 0.1 for _ in range(NARGS[ttype])]
