@@ -60,6 +60,21 @@ def bench_config(vs, **over):
     return vs.vs_config_default(**kw)
 
 
+def ncu_traffic(path=os.path.join(ROOT, "profiles", "r01s3_ncu_full_tcf.csv")):
+    """dram__bytes_read.sum + dram__bytes_write.sum of the committed ncu --set full capture of
+    one tcf_gemm_kernel launch inside the bench (bytes per launch), or None."""
+    import csv
+    scale = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}
+    try:
+        tot = 0.0
+        for m, unit, v in list(csv.reader(open(path)))[1:]:
+            if m in ("dram__bytes_read.sum", "dram__bytes_write.sum"):
+                tot += float(v) * scale.get(unit, 1)
+        return int(tot)
+    except (OSError, ValueError):
+        return None
+
+
 def peaks():
     p = os.path.join(ROOT, "MEASURED_PEAKS.json")
     if os.path.exists(p):
@@ -285,8 +300,13 @@ def roofline(log, groups, ms, world):
     # tensor-pipe busy fraction of the whole step: hardware MMA flops of every tensor-core
     # task / (step time x that version's peak), summed over versions
     frac_step = sum(3.0 * v["flops"] / tc_peak[k[1]][0] for k, v in per_tv.items() if k[1] in tc_peak) / (ms * 1e-3) / 1e12
+    traffic = ncu_traffic() if dom == "tcf_gemm_kernel" else None
     roof = {"bound": bound, "kernel": dom, "tasks": d["n"], "achieved": round(achieved, 2), "peak": round(peak, 1),
-            "unit": "TFLOP/s", "frac": round(achieved / peak, 4), "traffic": None, "peak_source": src,
+            "unit": "TFLOP/s", "frac": round(achieved / peak, 4), "traffic": traffic,
+            "traffic_note": ("DRAM bytes of one captured launch (ncu --set full, profiles/r01s3_ncu_full_tcf.csv: "
+                             "one SYRK b=1024 task; algorithmic 4 MiB form + 2.5 MiB C read + 2.5 MiB C written, "
+                             "C write-back happens after the kernel)") if traffic else None,
+            "peak_source": src,
             "how": "hardware MMA flops (3x the algorithmic flops of its tasks: 2b^3 matmul/gemm, b^3 syrk/trsm) of "
                    "every task this kernel ran in the timed steps / union of their device-recorded execution "
                    "intervals (%globaltimer, task_ctx.cuh)"}

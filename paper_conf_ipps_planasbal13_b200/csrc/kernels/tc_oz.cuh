@@ -22,17 +22,17 @@
 // 2^-7q and sA sB scalings exact; the 7-term sum is the only rounding besides C_in + .).
 //
 // Form byte layout, row-group size G = 128 (A role) or 64 (B role of an NT / NN product)
-// (Rp = R rounded up to 128, rows >= R are zero; K a multiple of 64):
-//   [kb = k / 64][row group r / G][slice s][row r % G][64 B], each 64-byte row in the UMMA
-//   canonical K-major SWIZZLE_64B layout (8-row atoms of 512 B, 16-byte chunk index XOR
-//   ((r >> 1) & 3)), then double sc[Rp] at byte S * Rp * K.  The 7 slices of one row group
-//   for one k-block are one contiguous block (56 KB for G = 128, 28 KB for G = 64), so a
+// (Rp = R rounded up to 128, rows >= R are zero; K a multiple of 64; KB = 32):
+//   [kb = k / KB][row group r / G][slice s][row r % G][KB bytes], each row in the UMMA
+//   canonical K-major SWIZZLE_32B layout (8-row atoms of 256 B, 16-byte chunk index XOR
+//   ((r >> 2) & 1)), then double sc[Rp] at byte S * Rp * K.  The 7 slices of one row group
+//   for one k-block are one contiguous block (28 KB for G = 128, 14 KB for G = 64), so a
 //   stage is filled by two bulk copies.
 //
 // GEMM (one 128 x 64 output tile per CTA, cta_group::1, UMMA M=128 N=64 K=32 kind::i8):
-//   warp 0     lane 0: per 64-wide k-block, the bulk copies of the stage (A: one 56 KB block;
-//              B: one 28 KB block, or 7 x 4 KB when B's form has G = 128, SYRK) onto the
-//              stage's full barrier (expect_tx).
+//   warp 0     lane 0: per 32-wide k-block, the bulk copies of the stage (A: one 28 KB block;
+//              B: one 14 KB block, or 7 x 2 KB when B's form has G = 128, SYRK) onto the
+//              stage's full barrier (expect_tx); 5 stages (210 KB) in flight.
 //   warp 1     TMEM allocator (512 columns; accumulator q at columns 64(q-2)) + MMA issuer:
 //              per 32-wide k-step 28 tcgen05.mma.kind::i8 (i = 1..7, j = 1..8-i),
 //              tcgen05.commit -> empty[s]; after the last k-block -> acc_full.
@@ -57,11 +57,15 @@ using tc::tc_fence_before;
 using tc::tmem_ld32;
 
 constexpr int S = 7;                     // slices
-constexpr int BM = 128, BN = 64, KB = 64;   // CTA tile; k-block = one 64-byte row of int8
-constexpr int SLA = BM * KB;             // 8 KB: one A slice of a stage
-constexpr int SLB = BN * KB;             // 4 KB: one B slice
-constexpr int STAGE = S * (SLA + SLB);   // 84 KB
-constexpr int STAGES = 2;
+// k-block = one KB-byte row of int8 per slice: 32 (SWIZZLE_32B rows, one MMA k-step per
+// stage, 42 KB stages, 5 in flight) or 64 (SWIZZLE_64B, 84 KB stages, 2 in flight: measured
+// load-latency bound)
+constexpr int BM = 128, BN = 64, KB = 32;   // CTA tile
+constexpr int SLA = BM * KB;             // one A slice of a stage
+constexpr int SLB = BN * KB;             // one B slice
+constexpr int STAGE = S * (SLA + SLB);
+constexpr int STAGES = KB == 64 ? 2 : 5;
+__host__ __device__ constexpr int swz(int r) { return KB == 64 ? ((r >> 1) & 3) : ((r >> 2) & 1); }
 constexpr int NTHREADS = 192;
 constexpr int EPI_LD = 33;               // padded row (doubles) of the epilogue staging
 constexpr int SMEM = STAGES * STAGE + 1024 + 256;
@@ -71,12 +75,12 @@ __host__ __device__ inline int rows_padded(int R) { return (R + 127) / 128 * 128
 __host__ __device__ inline size_t form_bytes(int R, int K) { return (size_t)S * rows_padded(R) * K + (size_t)rows_padded(R) * 8; }
 __host__ __device__ inline size_t slice_off(int Rp, int G, int kb, int s, int r, int chunk)
 {
-    return (((size_t)kb * (Rp / G) + r / G) * S + s) * G * 64 + (size_t)(r % G) * 64 + ((chunk ^ ((r >> 1) & 3)) << 4);
+    return (((size_t)kb * (Rp / G) + r / G) * S + s) * G * KB + (size_t)(r % G) * KB + ((chunk ^ swz(r)) << 4);
 }
 // byte offset of the 7-slice block of row group r0 / G for k-block kb
 __host__ __device__ inline size_t block_off(int Rp, int G, int kb, int r0)
 {
-    return ((size_t)kb * (Rp / G) + r0 / G) * S * G * 64;
+    return ((size_t)kb * (Rp / G) + r0 / G) * S * G * KB;
 }
 
 // Row scales: sc_r = 2^e with max|x_r| / sc_r in [1/2, 1).  Element (r, k) of the operand is
@@ -124,7 +128,7 @@ __global__ void __launch_bounds__(256) oz_slice_kernel(const double *__restrict_
         const int k = ch * 16 + i;
         t[i] = r < R ? __ldg(X + (int64_t)r * sr + (int64_t)k * sk) * inv : 0.0;   // inv = 2^-e: exact
     }
-    const int kb = ch >> 2, c = ch & 3;
+    const int kb = ch / (KB / 16), c = ch % (KB / 16);
 #pragma unroll 1
     for (int s = 0; s < S; s++) {
         uint32_t w[4];
@@ -151,16 +155,16 @@ __host__ __device__ constexpr uint32_t make_idesc_i8(int M, int N)
     return (2u << 4) | (1u << 7) | (1u << 10) | ((uint32_t)(N >> 3) << 17) | ((uint32_t)(M >> 4) << 24);
 }
 
-// UMMA shared-memory descriptor, K-major SWIZZLE_64B (layout type 4): 64-byte rows, 8-row
-// atoms of 512 B (SBO), LBO ignored for swizzled K-major, version 1.
-__device__ __forceinline__ uint64_t desc_sw64(uint32_t saddr)
+// UMMA shared-memory descriptor, K-major SWIZZLE_32B / 64B (layout type 6 / 4): KB-byte rows, 8-row
+// atoms (SBO = 8 * KB bytes), LBO ignored for swizzled K-major, version 1.
+__device__ __forceinline__ uint64_t desc_sw(uint32_t saddr)
 {
     uint64_t d = 0;
     d |= (uint64_t)((saddr & 0x3FFFF) >> 4);
     d |= (uint64_t)(16 >> 4) << 16;
-    d |= (uint64_t)(512 >> 4) << 32;
+    d |= (uint64_t)((8 * KB) >> 4) << 32;            // SBO: 8-row atom
     d |= (uint64_t)1 << 46;
-    d |= (uint64_t)4 << 61;
+    d |= (uint64_t)(KB == 64 ? 4 : 6) << 61;         // SWIZZLE_64B / SWIZZLE_32B
     return d;
 }
 
@@ -237,9 +241,9 @@ __global__ void __launch_bounds__(NTHREADS, 1)
                 if (GB == 64) {
                     bulk_g2s(st + S * SLA, Bf + block_off(RB, 64, kb, n0), S * SLB, &full[s]);
                 } else {   // rows n0 .. n0+63 of each slice of a 128-row group
-                    const uint8_t *bb = Bf + block_off(RB, 128, kb, n0) + (size_t)(n0 % 128) * 64;
+                    const uint8_t *bb = Bf + block_off(RB, 128, kb, n0) + (size_t)(n0 % 128) * KB;
                     for (int sl = 0; sl < S; sl++)
-                        bulk_g2s(st + S * SLA + sl * SLB, bb + (size_t)sl * 128 * 64, SLB, &full[s]);
+                        bulk_g2s(st + S * SLA + sl * SLB, bb + (size_t)sl * 128 * KB, SLB, &full[s]);
                 }
             }
         }
@@ -296,10 +300,10 @@ __global__ void __launch_bounds__(NTHREADS, 1)
                 for (int ks = 0; ks < KB / 32; ks++) {
 #pragma unroll
                     for (int i = 1; i <= S; i++) {
-                        const uint64_t da = desc_sw64(a0 + (i - 1) * SLA + ks * 32);
+                        const uint64_t da = desc_sw(a0 + (i - 1) * SLA + ks * 32);
 #pragma unroll
                         for (int j = 1; j <= S + 1 - i; j++) {
-                            const uint64_t db = desc_sw64(b0 + (j - 1) * SLB + ks * 32);
+                            const uint64_t db = desc_sw(b0 + (j - 1) * SLB + ks * 32);
                             const uint32_t first = (kb == 0 && ks == 0 && i == 1) ? 0u : 1u;
                             mma_i8(tmem + (uint32_t)((i + j - 2) * BN), da, db, idesc, first);
                         }
