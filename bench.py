@@ -20,6 +20,7 @@ of the same workload (this tier's reference arm).
 from __future__ import annotations
 
 import argparse
+import ctypes
 import json
 import math
 import os
@@ -176,7 +177,9 @@ class Workload:
             self.S.copy_(self.S0)
         if not self.host and sync:
             self.torch.cuda.current_stream().synchronize()
-        self.rt.vs_data_invalidate_n(self.ids)
+        if getattr(self, "_ids_arr", None) is None:
+            self._ids_arr = (ctypes.c_int64 * len(self.ids))(*self.ids)
+        self.rt.vs_data_invalidate_n(self._ids_arr)
 
     def submit(self):
         vs, rt = self.vs, self.rt

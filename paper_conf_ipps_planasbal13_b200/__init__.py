@@ -365,7 +365,7 @@ class Runtime:
         return self._ck(lib().vs_data_invalidate(self.h, d), "vs_data_invalidate")
 
     def vs_data_invalidate_n(self, ids):
-        a = _ids(list(ids))
+        a = ids if isinstance(ids, ctypes.Array) else _ids(list(ids))
         return self._ck(lib().vs_data_invalidate_n(self.h, ctypes.cast(a, c_void_p), len(a)), "vs_data_invalidate_n")
 
     def vs_dist_init(self, rank, nranks, shm_name=""):

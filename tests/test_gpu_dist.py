@@ -21,7 +21,7 @@ def _port():
     return p
 
 
-def _worker(rank, world, port, q):
+def _worker(rank, world, port, q, bench_cfg=False):
     import torch
     import torch.distributed as dist
 
@@ -40,7 +40,10 @@ def _worker(rank, world, port, q):
             dist.all_gather_object(out, obj)
             return out
 
-        rt = vs.Runtime(vs.vs_config_default(lam=1, slots_per_gpu=2, priority=1))
+        # run-ahead with type priority, or the launch configuration bench.py times (ready mode,
+        # bottom-level priority, 12 slots, group_hold: grouping is off across ranks)
+        rt = vs.Runtime(bench.bench_config(vs, lam=1) if bench_cfg else
+                        vs.vs_config_default(lam=1, slots_per_gpu=2, priority=1))
         shm = gather("/vsched_test_%d" % os.getpid() if rank == 0 else None)[0]
         if rank == 0:
             rt.vs_dist_init(rank, world, shm)
@@ -86,13 +89,14 @@ def _worker(rank, world, port, q):
         dist.destroy_process_group()
 
 
-def test_two_ranks_sharded_matmul_cholesky(gpu):
+@pytest.mark.parametrize("bench_cfg", [False, True])
+def test_two_ranks_sharded_matmul_cholesky(gpu, bench_cfg):
     import torch.multiprocessing as mp
     world = 2
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _port()
-    procs = [ctx.Process(target=_worker, args=(r, world, port, q)) for r in range(world)]
+    procs = [ctx.Process(target=_worker, args=(r, world, port, q, bench_cfg)) for r in range(world)]
     for p in procs:
         p.start()
     res = [q.get(timeout=600) for _ in range(world)]
