@@ -317,6 +317,18 @@ def roofline(log, groups, ms, world):
     return roof, frac_step, counts
 
 
+def config_json(args, world, mm_n=MM_N, mm_b=MM_B, ch_n=CH_N, ch_b=CH_B, with_mm=True, with_ch=True):
+    """The `config` of the JSON line (both arms print the same one)."""
+    return {"workload": ("cfg3+cfg4: tiled matmul N=%d b=%d + tiled Cholesky N=%d b=%d, fp32, versions "
+                         "simt_f32/tc_3xtf32/f64in_f32io/tc_3xf16, lambda=%d, %d slots/GPU" % (
+                             mm_n, mm_b, ch_n, ch_b, args.lam, args.slots)) if with_mm and with_ch else args.only,
+            "matmul_N": mm_n if with_mm else None, "cholesky_N": ch_n if with_ch else None,
+            "tile": mm_b, "lambda": args.lam, "slots_per_gpu": args.slots,
+            "parallelism": ("owner-computes 2D block-cyclic %dx%d, NVLink tile pulls" % rank_grid(world))
+            if world > 1 else "1 GPU",
+            "l2": "inputs larger than L2 (4 GiB + 4 GiB)", "regime": "warm (tables learned in warm-up)"}
+
+
 # ----------------------------------------------------------------------------- reference arm
 _CPU = {}
 
@@ -374,7 +386,7 @@ def run_reference(args, rank, world):
            "ms_per_step": round(1e3 * t / len(samples), 2), "higher_is_better": True,
            "scaling": "strong" if world > 1 else "weak", "vs_baseline": None, "dtype": "f64",
            "data": "synthetic (vsgen counter-based generator)",
-           "config": {"workload": "cfg3+cfg4 (bounded CPU sample)", "matmul_N": MM_N, "cholesky_N": CH_N},
+           "config": config_json(args, world),
            "cpu_baseline": {"value": round(gf, 3), "unit": "GFLOP/s", "cores": s0["cores"], "kind": "oracle",
                             "sample": sample},
            "e2e": {"value": round(gf, 3), "unit": "GFLOP/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
@@ -552,15 +564,7 @@ def main():
             "n_gpus": world, "steps": args.steps, "warmup": args.warmup, "ms_per_step": round(ms_step, 3),
             "higher_is_better": True, "scaling": "strong" if world > 1 else "weak", "vs_baseline": None, "dtype": "f32",
             "data": "synthetic (counter-based generator; U(-1,1) matmul operands, SPD A = S + 2.5 sqrt(N) I)",
-            "config": {"workload": ("cfg3+cfg4: tiled matmul N=%d b=%d + tiled Cholesky N=%d b=%d, fp32, versions "
-                                    "simt_f32/tc_3xtf32/f64in_f32io/tc_3xf16, lambda=%d, %d slots/GPU" % (
-                                        mm_n, mm_b, ch_n, ch_b, args.lam, args.slots)) if with_mm and with_ch else
-                       args.only,
-                       "matmul_N": mm_n if with_mm else None, "cholesky_N": ch_n if with_ch else None,
-                       "tile": mm_b, "lambda": args.lam, "slots_per_gpu": args.slots,
-                       "parallelism": ("owner-computes 2D block-cyclic %dx%d, NVLink tile pulls" % rank_grid(world))
-                       if world > 1 else "1 GPU",
-                       "l2": "inputs larger than L2 (4 GiB + 4 GiB)", "regime": "warm (tables learned in warm-up)"},
+            "config": config_json(args, world, mm_n, mm_b, ch_n, ch_b, with_mm, with_ch),
             "parts_gflop": {"matmul": MM_FLOPS(mm_n) / 1e9 if with_mm else 0,
                             "cholesky": CH_FLOPS(ch_n) / 1e9 if with_ch else 0},
             "cold_first_step_ms": round(cold_ms, 1),
