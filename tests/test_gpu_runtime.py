@@ -80,6 +80,37 @@ def test_matmul_host_data_copy_deps(gpu):
     rt.close()
 
 
+def test_host_data_bench_config_eager_writeback(gpu):
+    # host-homed tiles in the bench's launch configuration (ready mode, grouped launches): the
+    # final version of every written tile is copied home as soon as its last writer completes
+    # (eager flush), the rest of the graph still reading the GPU replica; results and Tx
+    # counters as with the flush at vs_wait_all
+    import torch
+
+    import bench
+    rt = vs.Runtime(bench.bench_config(vs, lam=1, slots_per_gpu=4))
+    mask = (1 << vs.VS_V_TC_3XTF32) | (1 << vs.VS_V_TC_3XF16)
+    A, B, C0, C = _matmul(rt, 1024, 256, mask=mask, host=True)
+    assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-5
+    st = rt.vs_stats()
+    assert st.output_tx_bytes == 16 * 256 * 256 * 4
+    rt.close()
+    rt = vs.Runtime(bench.bench_config(vs, lam=1, slots_per_gpu=4))
+    types = rt.vs_register_builtins(vs.VS_F32, mask)
+    N, b = 2048, 256
+    nt = N // b
+    S = vsgen.spd(12, N)
+    T = torch.from_numpy(vsgen.to_tiles(S, b)).pin_memory()
+    ids = {i * nt + j: rt.vs_data_register(T[i, j].data_ptr(), -1, b * b * 4) for i in range(nt) for j in range(i + 1)}
+    rt.vs_app_cholesky(types, nt, ids)
+    rt.vs_wait_all()
+    L = np.tril(vsgen.from_tiles(T.numpy()))
+    Lref, info = oracle.cholesky(S)
+    assert info == 0 and oracle.relF(L, Lref) <= 1e-5
+    assert rt.vs_stats().output_tx_bytes == len(ids) * b * b * 4   # every tile written once home
+    rt.close()
+
+
 def test_matmul_f64_family(gpu):
     rt = vs.Runtime(lam=1)
     mask = (1 << vs.VS_V_DFMA_F64) | (1 << vs.VS_V_DMMA_F64)
