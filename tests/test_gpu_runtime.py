@@ -111,6 +111,23 @@ def test_host_data_bench_config_eager_writeback(gpu):
     rt.close()
 
 
+def test_equally_critical_chains_run_concurrently(gpu):
+    # R33: in the bench configuration (bottom-level priority, critical-path streams) a lone
+    # matmul has 16 equally critical k-chains; they must run side by side, not queue on the
+    # two critical-path streams: some device-recorded task intervals overlap by 4 or more
+    import bench
+    rt = vs.Runtime(bench.bench_config(vs, lam=1))
+    _matmul(rt, 1024, 256, mask=(1 << vs.VS_V_TC_3XTF32) | (1 << vs.VS_V_TC_3XF16))
+    log = rt.vs_decision_log()
+    ev = sorted([(r[4], 1) for r in log] + [(r[5], -1) for r in log])
+    cur = best = 0
+    for _, d in ev:
+        cur += d
+        best = max(best, cur)
+    assert best >= 4, best
+    rt.close()
+
+
 def test_matmul_f64_family(gpu):
     rt = vs.Runtime(lam=1)
     mask = (1 << vs.VS_V_DFMA_F64) | (1 << vs.VS_V_DMMA_F64)
