@@ -190,6 +190,8 @@ class Workload:
             rt.vs_app_cholesky(self.types, self.ch_nt, self.iS)
 
     def step(self, barrier=None):
+        if barrier:
+            barrier()      # every rank finished the previous step: none still pulls a tile we restore
         # the restores run on the GPU while the host builds the step's task graph (vs_submit
         # only records tasks and dependences; nothing is issued before vs_wait_all)
         self.reset(sync=False)

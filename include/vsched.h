@@ -374,9 +374,14 @@ int vs_gen_tile(uint64_t seed, int64_t rows, int64_t cols, int dtype, int tile_b
  * registration) after the producing task's completion tag is visible: tags live in the
  * POSIX shared-memory segment shm_name (created by rank 0, which must call first; the
  * binding orders the calls with a barrier) registered with every rank's GPU, so the wait
- * is a stream memory operation on the device, with no host round trip.  Restrictions: run-
- * ahead mode; a rank never overwrites a datum another rank may still be copying (true of
- * vs_app_matmul / vs_app_cholesky with owner computes).  Must precede submissions. */
+ * is a stream memory operation on the device, with no host round trip.  Both decision modes
+ * work (ready mode parks a task until its remote predecessors' tags are visible).
+ * Restrictions: inside a graph a rank never overwrites a datum another rank may still be
+ * copying (true of vs_app_matmul / vs_app_cholesky with owner computes); between graphs the
+ * caller must not modify its owned data outside tasks (e.g. restore inputs) before every rank
+ * has returned from its vs_wait_all of the previous graph (a barrier), and other ranks must
+ * not read them before the modification is complete (a second barrier; see bench.py).  Must
+ * precede submissions. */
 int vs_dist_init(vs_rt rt, int rank, int nranks, const char *shm_name);
 /* Datum d is owned by rank `owner` (its pointer is then the owner's memory, opened with
  * vs_ipc_open); data registered without this call belong to the calling rank. */
