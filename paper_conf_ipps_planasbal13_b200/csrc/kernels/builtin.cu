@@ -218,24 +218,32 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
 struct TaskGroup {
     tcf::TcfGroup g;
 };
-int group_kind(int type, int version)
+int group_kind(int type, int version, int b)
 {
-    return (version == VS_V_TC_3XF16 && type != VS_T_POTRF) ? 1 : 0;
+    // a tile whose K needs several accumulation chunks (tc::kKChunk) runs as sequential
+    // launches, never inside a group
+    return (version == VS_V_TC_3XF16 && type != VS_T_POTRF && b <= tc::kKChunk) ? 1 : 0;
 }
 TaskGroup *group_new() { return new TaskGroup(); }
 void group_free(TaskGroup *g) { delete g; }
 int group_size(const TaskGroup *g) { return g->g.n; }
 int group_ctas(const TaskGroup *g) { return g->g.ctas; }
-int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const TaskCtx &ctx)
+// the K-chunk [k0, k0 + kc) of one tc_3xf16 task (kc < 0: all of K)
+static int group_add_chunk(TaskGroup *g, int type, int b, void *const *p, const TaskCtx &ctx, int k0, int kc)
 {
-    if (!group_kind(type, version)) return -1;
     switch (type) {   // p[i] tiles, p[np + i] forms (np = 3 / 2 / 2)
-    case VS_T_MATMUL: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, false, false, ctx);
-    case VS_T_GEMM_NT: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, true, false, ctx);
-    case VS_T_SYRK: return tcf::tcf_group_add(g->g, b, b, b, p[2], p[2], (float *)p[1], b, true, true, ctx);
-    case VS_T_TRSM: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[2], (float *)p[1], b, false, false, ctx, true);
+    case VS_T_MATMUL: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, false, false, ctx, false, k0, kc);
+    case VS_T_GEMM_NT: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, true, false, ctx, false, k0, kc);
+    case VS_T_SYRK: return tcf::tcf_group_add(g->g, b, b, b, p[2], p[2], (float *)p[1], b, true, true, ctx, false, k0, kc);
+    case VS_T_TRSM:   // X = B inv(L)^T: C_in not read by the first chunk
+        return tcf::tcf_group_add(g->g, b, b, b, p[3], p[2], (float *)p[1], b, false, false, ctx, k0 == 0, k0, kc);
     }
     return -1;
+}
+int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const TaskCtx &ctx)
+{
+    if (!group_kind(type, version, b)) return -1;
+    return group_add_chunk(g, type, b, p, ctx, 0, -1);
 }
 int group_launch(TaskGroup *g, cudaStream_t s) { return tcf::tcf_group_launch(g->g, s); }
 
@@ -253,10 +261,14 @@ int run_oz(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
 // tc_3xf16: p[] holds the split forms of the in-operands (builtin_operand_form)
 int run_f16(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
 {
-    TaskGroup g;
-    const int r = group_add(&g, type, VS_V_TC_3XF16, b, p, ctx);
-    if (r <= 0) return r;
-    return group_launch(&g, s);
+    if (type == VS_T_POTRF) return -1;
+    for (int k0 = 0; k0 < b; k0 += tc::kKChunk) {   // accumulation accuracy: see tc::tc_gemm
+        TaskGroup g;
+        const int r = group_add_chunk(&g, type, b, p, ctx, k0, b - k0 < tc::kKChunk ? b - k0 : tc::kKChunk);
+        if (r <= 0) return r;
+        if (group_launch(&g, s)) return -1;
+    }
+    return 0;
 }
 }  // namespace
 

@@ -63,7 +63,7 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s);
 // group_add() (ptrs as for launch_builtin, ctx of the task; returns the task's CTA count,
 // or -1 if it does not fit / is unsupported) and launched by group_launch().
 struct TaskGroup;
-int group_kind(int type, int version);
+int group_kind(int type, int version, int b);
 TaskGroup *group_new();
 void group_free(TaskGroup *g);
 int group_size(const TaskGroup *g);

@@ -305,7 +305,8 @@ __device__ __forceinline__ void mma_f16(uint32_t tmem_d, uint64_t adesc, uint64_
 // flags: bit 0 = negate (s = -1), bit 1 = LOWER (only tiles with j <= i exist, and the
 // diagonal tiles store j <= i), bit 2 = BETA0 (C = s A B'^T: C_in is not read).  The task's CTAs are [tile0, tile0 + ntiles) of the grid.
 struct TcfTask {
-    const uint8_t *As, *Bs;
+    const uint8_t *As, *Bs;          // split forms, advanced to the task's first k-block
+    const float *sa, *sb;            // their row scales 2^-e (at the end of the full forms)
     float *C;
     int M, N, K, ldc;
     int flags, tile0, ntiles, tiles_n;
@@ -475,8 +476,8 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         const int q = warp & 3, eh = (warp - 2) >> 2;   // TMEM lane quarter, column half
         float *stg = reinterpret_cast<float *>(smem) + (warp - 2) * 32 * EPI_LD;   // this warp's 32 x 128 block
         const int ccol = eh * 128 + lane * 4;            // this lane's 4 columns in the store phase
-        const float *sav = reinterpret_cast<const float *>(As + (size_t)RA * K * 4) + m0;
-        const float4 sb = __ldg(reinterpret_cast<const float4 *>(reinterpret_cast<const float *>(Bs + (size_t)RB * K * 4) + n0 + ccol));
+        const float *sav = tk.sa + m0;
+        const float4 sb = __ldg(reinterpret_cast<const float4 *>(tk.sb + n0 + ccol));
         const bool BETA0 = (tk.flags >> 2) & 1;   // C = s A B'^T (C_in not read)
         if (!BETA0 && !ghost) {   // C_in into L2 while the main loop runs (LSU prefetches: bulk prefetches
             // would occupy the TMA unit that feeds the operands): thread t -> tile row t, its 1 KB
@@ -586,22 +587,28 @@ inline bool tcf_pair()
     return v != 0;
 }
 
+// K-chunk [k0, k0 + kc) of a GEMM whose split forms have K columns (k0, kc multiples of 32;
+// kc = K: the whole product)
 inline int tcf_group_add(TcfGroup &g, int M, int N, int K, const void *As, const void *Bs, float *C, int ldc,
-                         bool neg, bool lower, TaskCtx ctx, bool beta0 = false)
+                         bool neg, bool lower, TaskCtx ctx, bool beta0 = false, int k0 = 0, int kc = -1)
 {
     if (M <= 0 || N <= 0) return 0;
-    if (K % BK || ldc % 4 || g.n >= kMaxGroup || (lower && M != N)) return -1;
+    if (kc < 0) kc = K;
+    if (K % BK || k0 % BK || kc % BK || k0 + kc > K || ldc % 4 || g.n >= kMaxGroup || (lower && M != N)) return -1;
     const int tm = (M + BT - 1) / BT, tn = (N + BT - 1) / BT;
     int nt = lower ? tm * (tm + 1) / 2 : tm * tn;
     if (tcf_pair()) {   // two CTAs per pair of tiles in a row (kernel comment): rows hold ceil(tn/2)
         nt = 0;         // pairs, row bi of a LOWER task bi/2 + 1
         for (int bi = 0; bi < tm; bi++) nt += 2 * (lower ? bi / 2 + 1 : (tn + 1) / 2);
     }
+    const int RA = split_rows_padded(M), RB = split_rows_padded(N);
     TcfTask &t = g.t[g.n++];
-    t.As = (const uint8_t *)As;
-    t.Bs = (const uint8_t *)Bs;
+    t.As = (const uint8_t *)As + (size_t)(k0 / BK) * RA * 128;
+    t.Bs = (const uint8_t *)Bs + (size_t)(k0 / BK) * RB * 128;
+    t.sa = reinterpret_cast<const float *>((const uint8_t *)As + (size_t)RA * K * 4);
+    t.sb = reinterpret_cast<const float *>((const uint8_t *)Bs + (size_t)RB * K * 4);
     t.C = C;
-    t.M = M; t.N = N; t.K = K; t.ldc = ldc;
+    t.M = M; t.N = N; t.K = kc; t.ldc = ldc;
     t.flags = (neg ? 1 : 0) | (lower ? 2 : 0) | (beta0 ? 4 : 0);
     t.tile0 = g.ctas;
     t.ntiles = nt;
@@ -684,10 +691,14 @@ template <bool NEG, bool LOWER>
 inline int tcf_gemm(int M, int N, int K, const void *As, const void *Bs, float *C, int ldc, cudaStream_t s,
                     const TaskCtx &ctx = TaskCtx())
 {
-    TcfGroup g;
-    const int r = tcf_group_add(g, M, N, K, As, Bs, C, ldc, NEG, LOWER, ctx);
-    if (r <= 0) return r;
-    return tcf_group_launch(g, s);
+    for (int k0 = 0; k0 < K; k0 += tc::kKChunk) {   // accumulation accuracy: see tc::tc_gemm
+        TcfGroup g;
+        const int r = tcf_group_add(g, M, N, K, As, Bs, C, ldc, NEG, LOWER, ctx, false, k0,
+                                    K - k0 < tc::kKChunk ? K - k0 : tc::kKChunk);
+        if (r <= 0) return r;
+        if (tcf_group_launch(g, s)) return -1;
+    }
+    return 0;
 }
 
 }  // namespace tcf

@@ -303,3 +303,20 @@ def test_tc_3xf16_forms_follow_writes_and_invalidation(gpu):
     assert oracle.relF(vsgen.from_tiles(tC.cpu().numpy()), A2.astype(np.float64) @ B) <= 1e-5
     assert rt.vs_stats().forms_built == n1 + nt * nt
     rt.close()
+
+
+def test_empty_graph_and_single_tile_problems(gpu):
+    # degenerate graphs: vs_wait_all with nothing submitted, a 1x1x1 tiled matmul (one task)
+    # and a one-tile Cholesky (a single potrf) through the runtime, every f32 version enabled
+    rt = vs.Runtime(lam=1)
+    rt.vs_wait_all()
+    assert rt.vs_stats().tasks_completed == 0
+    A, B, C0, C = _matmul(rt, 256, 256, mask=F32_MASK | (1 << vs.VS_V_TC_3XF16))
+    assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-5
+    rt.close()
+    rt = vs.Runtime(lam=1)
+    S, L = _cholesky(rt, 256, 256)
+    Lref, info = oracle.cholesky(S)
+    assert info == 0 and oracle.relF(L, Lref) <= 1e-5
+    assert rt.vs_stats().tasks_completed == 1
+    rt.close()

@@ -228,3 +228,30 @@ def test_potrf_integer_L0_exact_and_info(gpu, version):
     info.zero_()
     _run(vs.VS_T_POTRF, version, b, [bad], info)
     assert int(info.item()) == 70
+
+
+# ------------------------------------------------------------------ edge cases
+@pytest.mark.parametrize("version", [vs.VS_V_TC_3XF16, vs.VS_V_TC_3XTF32])
+def test_max_tile_4096_sampled_rows(gpu, version):
+    # the largest tile the built-in versions accept (b = 4096, 64 MiB per fp32 tile): C = C0 + A B
+    # and C0 - A B^T, checked on sampled rows the oracle computes one by one (first, last, a
+    # 256-row group boundary, the middle).  K = 4096 is accumulated in chunks of 1024 (R34):
+    # before, tc_3xtf32 measured relF 2.9e-5 and tc_3xf16 1.4e-5 here
+    b = 4096
+    A, B, C0 = (vsgen.uniform(800 + i, b, b) for i in range(3))
+    rows = [0, 255, 256, 2047, 4095]
+    (_, _, C) = _run(vs.VS_T_MATMUL, version, b, [A, B, C0])
+    ref = oracle.matmul(A[rows], B, C0[rows])
+    assert oracle.relF(C[rows], ref) <= 1e-5
+    (_, _, G) = _run(vs.VS_T_GEMM_NT, version, b, [A, B, C0])
+    ref = oracle.matmul(-A[rows], np.ascontiguousarray(B.T), C0[rows])   # C0 - A B^T (negation exact)
+    assert oracle.relF(G[rows], ref) <= 1e-5
+
+
+@pytest.mark.parametrize("b", [0, 32, 96, 8192])
+def test_unsupported_tile_sizes_rejected(gpu, b):
+    # b must be a positive multiple of 64 up to 4096: anything else is VS_E_INVAL, no launch
+    torch = _torch()
+    t = torch.zeros(max(1, min(b, 128)) ** 2, device="cuda")
+    with pytest.raises(vs.VSError):
+        vs.vs_tile_run(vs.VS_T_MATMUL, vs.VS_V_TC_3XTF32, b, [t.data_ptr()] * 3)
