@@ -255,3 +255,22 @@ def test_unsupported_tile_sizes_rejected(gpu, b):
     t = torch.zeros(max(1, min(b, 128)) ** 2, device="cuda")
     with pytest.raises(vs.VSError):
         vs.vs_tile_run(vs.VS_T_MATMUL, vs.VS_V_TC_3XTF32, b, [t.data_ptr()] * 3)
+
+
+@pytest.mark.parametrize("ttype", ["MATMUL", "GEMM_NT"])
+def test_oz_i8_f64_full_53bit_inputs(gpu, ttype):
+    # the generator's values have 24-bit mantissas, which 7 int8 slices (49 bits) hold exactly;
+    # full-precision fp64 inputs exercise the slice truncation and the dropped slice products:
+    # relF within the fp64 gate and the componentwise bound of the scheme (tc_oz.cuh)
+    b = 256
+    rng = np.random.default_rng(11)
+    A, B, C0 = (rng.standard_normal((b, b)) for _ in range(3))
+    t = getattr(vs, "VS_T_" + ttype)
+    (_, _, C) = _run(t, vs.VS_V_OZ_I8_F64, b, [A, B, C0])
+    Bop = B if ttype == "MATMUL" else B.T
+    ref = oracle.matmul(A, np.ascontiguousarray(Bop), C0) if ttype == "MATMUL" else oracle.gemm_nt(A, B, C0)
+    assert oracle.relF(C, ref) <= 1e-12
+    bound = 2.0 ** -44 * (np.abs(A) @ np.abs(Bop)) + b * 2.0 ** -45 * np.max(np.abs(A), axis=1, keepdims=True) * \
+        np.max(np.abs(Bop), axis=0, keepdims=True)
+    assert np.all(np.abs(C - ref) <= bound)
+    assert oracle.relF(C, ref) > 0.0     # not exact: the truncation is really exercised
