@@ -296,18 +296,24 @@ __global__ void __launch_bounds__(NTHREADS, 1)
             tc_fence_after();
             if (lane == 0) {
                 const uint32_t a0 = smem_u32(smem + s * STAGE), b0 = a0 + S * SLA;
+                // descriptors of the stage's slices computed once: the start-address field is
+                // linear (addr >> 4, no carry below 256 KB), so slice i is the base + a constant;
+                // 28 MMAs of N = 64 (32 clk each) leave few issue slots per MMA
+                const uint64_t dA0 = desc_sw(a0), dB0 = desc_sw(b0);
 #pragma unroll
                 for (int ks = 0; ks < KB / 32; ks++) {
+                    uint64_t da[S], db[S];
 #pragma unroll
-                    for (int i = 1; i <= S; i++) {
-                        const uint64_t da = desc_sw(a0 + (i - 1) * SLA + ks * 32);
-#pragma unroll
-                        for (int j = 1; j <= S + 1 - i; j++) {
-                            const uint64_t db = desc_sw(b0 + (j - 1) * SLB + ks * 32);
-                            const uint32_t first = (kb == 0 && ks == 0 && i == 1) ? 0u : 1u;
-                            mma_i8(tmem + (uint32_t)((i + j - 2) * BN), da, db, idesc, first);
-                        }
+                    for (int i = 0; i < S; i++) {
+                        da[i] = dA0 + (uint64_t)((i * SLA + ks * 32) >> 4);
+                        db[i] = dB0 + (uint64_t)((i * SLB + ks * 32) >> 4);
                     }
+                    const uint32_t f0 = (kb == 0 && ks == 0) ? 0u : 1u;
+#pragma unroll
+                    for (int i = 1; i <= S; i++)
+#pragma unroll
+                        for (int j = 1; j <= S + 1 - i; j++)
+                            mma_i8(tmem + (uint32_t)((i + j - 2) * BN), da[i - 1], db[j - 1], idesc, i == 1 ? f0 : 1u);
                 }
                 tc::mma_commit(&empty[s]);
                 if (kb == nk - 1) tc::mma_commit(acc_full);
