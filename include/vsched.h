@@ -168,7 +168,10 @@ typedef struct {
  * run-ahead, live timing, flush.  Environment overrides applied by vs_create (L277-288):
  * VS_LAMBDA, VS_SLOTS, VS_POLICY(=versioning|fixed:<v>), VS_LEARNING(=hold|rr),
  * VS_MODE(=runahead|ready), VS_LOOKAHEAD(=n), VS_PRIORITY(=0|1|2), VS_QDEPTH(=d), VS_GROUP_HOLD(=0|1),
- * VS_GROUP(=tasks per grouped launch), VS_GROUP_US. */
+ * VS_GROUP(=tasks per grouped launch), VS_GROUP_US.  Runtime options outside vs_config:
+ * VS_TRACKER(=events|memops) dependence tracker on one GPU, VS_GROUP_DIST(=0|1, default 1)
+ * grouped launches in a multi-rank job, VS_PREFETCH(=n, default 0) input-prefetch window on one
+ * GPU, VS_TCF_PAIR(=0|1, default 1) CTA-pair variant of the tc_3xf16 GEMM. */
 void vs_config_default(vs_config *cfg);
 
 /* Create a runtime.  *out receives an opaque handle owning scheduler state, DAG,
