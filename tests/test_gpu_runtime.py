@@ -320,3 +320,27 @@ def test_empty_graph_and_single_tile_problems(gpu):
     assert info == 0 and oracle.relF(L, Lref) <= 1e-5
     assert rt.vs_stats().tasks_completed == 1
     rt.close()
+
+
+def test_multi_kernel_tasks_b2048_through_runtime(gpu):
+    # b = 2048 tensor-core tasks run as two K-chunk launches each (R34): a task completes only
+    # when its last kernel reported through the completion ring (nkern = 2).  A 2x2x2 tiled
+    # matmul (N = 4096) with tc_3xtf32 and tc_3xf16, results on sampled rows against the oracle
+    import bench
+    torch = _torch()
+    rt = vs.Runtime(bench.bench_config(vs, lam=1, slots_per_gpu=4))
+    N, b = 4096, 2048
+    nt = N // b
+    types = rt.vs_register_builtins(vs.VS_F32, (1 << vs.VS_V_TC_3XTF32) | (1 << vs.VS_V_TC_3XF16))
+    A, B = vsgen.uniform(31, N, N), vsgen.uniform(1031, N, N)
+    tA, tB, tC = (_tiles_dev(x, b) for x in (A, B, np.zeros((N, N), np.float32)))
+    ia, ib, ic = (_register_tiles(rt, t) for t in (tA, tB, tC))
+    rt.vs_app_matmul(types[vs.VS_T_MATMUL], nt, nt, nt, ia, ib, ic)
+    rt.vs_wait_all()
+    torch.cuda.synchronize()
+    C = vsgen.from_tiles(tC.cpu().numpy())
+    rows = [0, 2047, 2048, 4095]
+    assert oracle.relF(C[rows], oracle.matmul(A[rows], B)) <= 1e-5
+    st = rt.vs_stats()
+    assert st.tasks_completed == 8 and st.kernel_launches >= 16
+    rt.close()
