@@ -42,10 +42,10 @@ SEED_MM, SEED_CH = 3, 4
 # runtime configuration the bench times (env VS_SLOTS / VS_PRIORITY / VS_QDEPTH override):
 # lambda 3, 12 workers (streams) per GPU, decisions when predecessors completed (ready mode:
 # no cross-stream waits, so no stream is blocked at its head), NEXT-4 bottom-level priority
-# with a real queue cap of 2 grouped launches per worker, grouped launches of up to 8
+# with a real queue cap of 1 grouped launch (8 tasks) per worker, grouped launches of up to 8
 # tc_3xf16 tasks held up to 200 us while their stream still runs a kernel (group_hold),
 # critical-path tasks on their own greatest-priority streams
-RT_DEFAULTS = dict(lam=3, slots=12, priority=2, qdepth=2, group=8, mode="ready", hold=1, group_us=200)
+RT_DEFAULTS = dict(lam=3, slots=12, priority=2, qdepth=1, group=8, mode="ready", hold=1, group_us=200)
 F32_VERSIONS_MASK = 0b100111  # simt_f32 | tc_3xtf32 | f64in_f32io | tc_3xf16 (gemm-type tasks)
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
