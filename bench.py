@@ -89,6 +89,14 @@ def rank_grid(nranks):
     return {1: (1, 1), 2: (1, 2), 4: (2, 2), 8: (2, 4)}.get(nranks, (1, nranks))
 
 
+def rank_device(local_rank, ndev):
+    """CUDA ordinal of this rank (one process per GPU): LOCAL_RANK; ranks beyond the visible
+    devices time-share them round-robin (only used to test multi-rank runs on one GPU).  The
+    runtime's gpu 0 is this device (vs_config.device_base), so its streams, replicas and
+    kernels live on the rank's own GPU."""
+    return local_rank % max(1, ndev)
+
+
 def tile_owner(i, j, nranks):
     pr, pc = rank_grid(nranks)
     return (i % pr) * pc + (j % pc)
@@ -434,7 +442,7 @@ def main():
     import torch
     import paper_conf_ipps_planasbal13_b200 as vs
     ndev = torch.cuda.device_count()
-    torch.cuda.set_device(local % max(1, ndev))
+    torch.cuda.set_device(rank_device(local, ndev))
     dist = None
     if world > 1:
         import torch.distributed as dist
@@ -456,9 +464,9 @@ def main():
     prio, qdepth = args.priority, args.qdepth
     look = int(os.environ.get("VS_LOOKAHEAD", "0"))
     mode = 1 if args.mode == "ready" else 0          # VS_MODE_READY / VS_MODE_RUNAHEAD
-    cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=0, replay=1 if args.replay else 0,
-                               priority=prio, lookahead=look, queue_depth=qdepth, group_tasks=args.group, mode=mode,
-                               group_hold=args.hold, group_wait_us=args.group_us)
+    cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=rank_device(local, ndev),
+                               replay=1 if args.replay else 0, priority=prio, lookahead=look, queue_depth=qdepth,
+                               group_tasks=args.group, mode=mode, group_hold=args.hold, group_wait_us=args.group_us)
     rt = vs.Runtime(cfg)
     if world > 1:
         shm = gather("/vsched_%d_%d" % (os.getpid(), int(time.time())) if rank == 0 else None)[0]

@@ -116,7 +116,9 @@ typedef struct {
     int slots_per_gpu; /* S workers (streams) per GPU (R16); S=1 is paper-literal */
     int lambda;        /* learning runs per version (L438-440, L461); default 3 (R10) */
     int policy;        /* VS_POLICY_VERSIONING | VS_POLICY_FIXED */
-    int fixed_version; /* version index used by VS_POLICY_FIXED */
+    int fixed_version; /* version index used by VS_POLICY_FIXED (a per-type index, see
+                          vs_register_builtins); vs_submit returns VS_E_INVAL for a type that
+                          has no runnable version of that index */
     int learning;      /* VS_LEARN_HOLD | VS_LEARN_RR */
     int mode;          /* VS_MODE_RUNAHEAD | VS_MODE_READY */
     int replay;        /* 1: the scheduler takes run times from the timing table, not from
@@ -197,16 +199,25 @@ typedef int (*vs_launch_fn)(void *const *dev_ptrs, const int64_t *bytes, int nar
 
 /* Add a version to a type ("implements(main)", Fig 4).  All versions share the
  * type's parameters and modes (L306-308).  gpu_mask bit g = runnable on runtime gpu g
- * (the device clause, L339-345).  *out = version index within the type (0,1,...). */
+ * (the device clause, L339-345); a mask naming no configured gpu is VS_E_INVAL.
+ * *out = version index within the type (0,1,...).  Versions must be added before the first
+ * submission (VS_E_STATE after it).  The runtime times a user version with a CUDA event pair
+ * around fn on the worker's stream (R17). */
 int vs_version_add(vs_rt rt, vs_type_id type, const char *name, uint32_t gpu_mask,
                    vs_launch_fn fn, void *user, vs_version_id *out);
 
-/* Register the five built-in tile task types for dtype (VS_F32: versions SIMT_F32,
- * TC_3XTF32, F64IN_F32IO, TC_3XF16 (MATMUL/GEMM_NT/SYRK only); VS_F64: DFMA_F64,
- * DMMA_F64), keeping the versions whose
- * bit is set in version_mask (bit = VS_V_*).  out_types[VS_T_*] receives the type ids;
- * version index order inside each type follows increasing VS_V_* id.  Runnable on
- * every gpu.  Errors: VS_E_INVAL if no version of dtype is selected. */
+/* Register the five built-in tile task types for dtype, keeping the versions whose bit is
+ * set in version_mask (bit = VS_V_*).  Versions each type actually gets:
+ *   VS_F32: SIMT_F32, TC_3XTF32, F64IN_F32IO for all five types; TC_3XF16 for MATMUL,
+ *           GEMM_NT, SYRK and TRSM (by inverse, R31) — not POTRF.
+ *   VS_F64: DFMA_F64, DMMA_F64 for all five types; OZ_I8_F64 for MATMUL, GEMM_NT, SYRK —
+ *           not POTRF / TRSM.
+ * out_types[VS_T_*] receives the type ids.  Version INDICES are per type: inside each type
+ * the kept versions are numbered 0, 1, ... in increasing VS_V_* order, skipping those the type
+ * does not get, so the same index may name different versions in different types (e.g. with
+ * every f32 version selected, index 3 is TC_3XF16 for MATMUL but does not exist for POTRF);
+ * vs_version_name() maps an index back to its name.  Runnable on every gpu.
+ * Errors: VS_E_INVAL if no version of dtype is selected. */
 int vs_register_builtins(vs_rt rt, int dtype, uint32_t version_mask,
                          vs_type_id out_types[VS_NUM_BUILTIN_TYPES]);
 
@@ -222,7 +233,8 @@ int vs_data_register(vs_rt rt, void *ptr, int device, int64_t bytes, vs_data_id 
  * VS_E_STATE if a task writing d is still in flight. */
 int vs_data_invalidate(vs_rt rt, vs_data_id d);
 
-/* vs_data_invalidate of ids[0..n-1] (one call for a whole matrix of tiles); stops at, and
+/* (Both invalidation calls first wait for copies back to the host that are still in flight.)
+ * vs_data_invalidate of ids[0..n-1] (one call for a whole matrix of tiles); stops at, and
  * returns the error of, the first failing id. */
 int vs_data_invalidate_n(vs_rt rt, const vs_data_id *ids, int64_t n);
 
@@ -234,8 +246,12 @@ int vs_submit(vs_rt rt, vs_type_id type, const vs_data_id *args, int nargs,
               const void *scalars, size_t nscalar, vs_task_id *out);
 
 /* ----------------------------------------------------------- waits (a15) */
+/* Every wait (and vs_create / vs_destroy) leaves the calling thread's current CUDA device
+ * as it found it. */
 int vs_wait_all(vs_rt rt);          /* taskwait: all tasks, then flush to home */
-int vs_wait_all_noflush(vs_rt rt);  /* taskwait noflush (L267-270) */
+int vs_wait_all_noflush(vs_rt rt);  /* taskwait noflush (L267-270): all tasks; written data
+                                       stay on the devices (copies back to the host that the
+                                       runtime had already started are completed first) */
 int vs_wait_on(vs_rt rt, vs_data_id d); /* taskwait on(d): d's last writer done; d valid at home */
 
 /* ---------------------------------------------------------------- statistics */
@@ -329,7 +345,7 @@ int vs_app_cholesky(vs_rt rt, const vs_type_id types[VS_NUM_BUILTIN_TYPES], int 
  * the runtime (used by parity tests and the smoke check).  ptrs as in VS_T_* order,
  * device pointers, tiles b x b contiguous.  dinfo: device int32 receiving potrf's info
  * (may be NULL for other types).  Returns VS_E_INVAL for an unknown (type, version)
- * or an unsupported b (b must be a multiple of 32, 32 <= b <= 4096). */
+ * or an unsupported b (b must be a multiple of 64, 64 <= b <= 4096). */
 int vs_tile_run(int type, int version, int b, void *const *ptrs, int *dinfo, void *stream);
 
 /* Derived operand forms (reading R30).  vs_operand_form returns the form (0 = the tile
@@ -394,6 +410,10 @@ int vs_data_set_owner(vs_rt rt, vs_data_id d, int owner);
 int vs_ipc_export(const void *dev_ptr, unsigned char handle[64], uint64_t *offset);
 int vs_ipc_open(const unsigned char handle[64], uint64_t offset, void **dev_ptr);
 int vs_ipc_close(void *base_ptr);
+
+/* CUDA ordinal of runtime gpu g (device_base + g), VS_E_INVAL if g is not a gpu of rt (SIM
+ * runtimes have none).  One process per GPU: every rank's runtime drives its own device. */
+int vs_gpu_ordinal(vs_rt rt, int g);
 
 /* Library build information (never NULL). */
 const char *vs_build_info(void);

@@ -129,6 +129,7 @@ def lib():
         "vs_form_make": (c_int, [c_int, c_int, c_void_p, c_void_p, c_void_p]),
         "vs_tile_run_prepared": (c_int, [c_int, c_int, c_int, POINTER(c_void_p), c_void_p, c_void_p]),
         "vs_decision_issue_ns": (c_int, [rt, POINTER(c_int64), c_int64, POINTER(c_int64)]),
+        "vs_gpu_ordinal": (c_int, [rt, c_int]),
     }
     for name, (res, args) in sig.items():
         f = getattr(L, name)
@@ -145,7 +146,7 @@ EXPORTED = ["vs_config_default", "vs_create", "vs_destroy", "vs_last_error", "vs
             "vs_replay_set", "vs_app_matmul", "vs_app_cholesky", "vs_tile_run", "vs_gen_uniform", "vs_gen_spd",
             "vs_build_info", "vs_gen_tile", "vs_dist_init", "vs_data_set_owner", "vs_ipc_export", "vs_ipc_open",
             "vs_ipc_close", "vs_data_invalidate", "vs_data_invalidate_n", "vs_operand_form", "vs_form_bytes", "vs_form_make",
-            "vs_tile_run_prepared", "vs_decision_issue_ns"]
+            "vs_tile_run_prepared", "vs_decision_issue_ns", "vs_gpu_ordinal"]
 
 
 def _ids(seq, ctype=c_int64):
@@ -367,6 +368,12 @@ class Runtime:
     def vs_data_invalidate_n(self, ids):
         a = ids if isinstance(ids, ctypes.Array) else _ids(list(ids))
         return self._ck(lib().vs_data_invalidate_n(self.h, ctypes.cast(a, c_void_p), len(a)), "vs_data_invalidate_n")
+
+    def vs_gpu_ordinal(self, g=0):
+        r = lib().vs_gpu_ordinal(self.h, g)
+        if r < 0:
+            raise VSError(r, "vs_gpu_ordinal(%d)" % g)
+        return r
 
     def vs_dist_init(self, rank, nranks, shm_name=""):
         return self._ck(lib().vs_dist_init(self.h, rank, nranks, shm_name.encode()), "vs_dist_init")

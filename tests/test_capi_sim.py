@@ -358,3 +358,35 @@ def test_next4_bottom_level_with_queue_depth_shortens_the_mixed_makespan():
         got, _ = _mixed(8, 16, 3, 6, BENCH_US, model=False, **kw)
         span[key] = max(r[5] for r in got)
     assert span["next4"] < span["paper"]
+
+
+def test_fixed_policy_version_checked_per_type():
+    """VS_POLICY_FIXED indexes each type's own version list: an index that a type does not have
+    is rejected at submission instead of reading past its versions."""
+    rt = _sim(policy=vs.VS_POLICY_FIXED, fixed_version=2)
+    t3 = rt.vs_type_create("T3", [vs.VS_INOUT])
+    t2 = rt.vs_type_create("T2", [vs.VS_INOUT])
+    for v in range(3):
+        rt.vs_version_add(t3, "v%d" % v, ALL)
+    for v in range(2):
+        rt.vs_version_add(t2, "v%d" % v, ALL)
+    d = rt.vs_data_register(_fake_ptr(0, 4096), 0, 4096)
+    rt.vs_replay_set(t3, 4096, 2, 1000)
+    rt.vs_submit(t3, [d])
+    with pytest.raises(vs.VSError) as e:
+        rt.vs_submit(t2, [d])
+    assert e.value.code == vs.VS_E_INVAL and "fixed version 2" in rt.vs_last_error()
+    rt.vs_wait_all()
+    assert [r[1] for r in rt.vs_decision_log()] == [2]
+
+
+def test_version_mask_must_name_a_configured_gpu():
+    rt = _sim(n_gpus=2)
+    t = rt.vs_type_create("T", [vs.VS_INOUT])
+    with pytest.raises(vs.VSError) as e:
+        rt.vs_version_add(t, "nowhere", 1 << 2)   # only gpus 0 and 1 exist
+    assert e.value.code == vs.VS_E_INVAL
+    with pytest.raises(vs.VSError):
+        rt.vs_submit(t, [rt.vs_data_register(_fake_ptr(0, 4096), 0, 4096)])   # no version at all
+    rt.vs_version_add(t, "gpu1", 1 << 1)
+    assert rt.vs_submit(t, [rt.vs_data_register(_fake_ptr(0, 4096), 0, 4096)]) == 0

@@ -98,3 +98,12 @@ def test_owner_computes_partition_gloo(world):
         i, j = writes[t]
         assert rank == bench.tile_owner(i, j, world)
     assert len({r for r in executed.values()}) == world   # both ranks work
+
+
+def test_rank_device_binding():
+    """bench.py binds rank r (LOCAL_RANK) to CUDA device r: torch's current device and the
+    runtime's vs_config.device_base both come from bench.rank_device (§8(e))."""
+    assert [bench.rank_device(r, 8) for r in range(8)] == list(range(8))
+    assert [bench.rank_device(r, 1) for r in range(4)] == [0, 0, 0, 0]   # time-sharing one GPU (tests)
+    src = open(bench.__file__).read()
+    assert "device_base=rank_device(local, ndev)" in src and "set_device(rank_device(local, ndev))" in src

@@ -33,7 +33,8 @@ def _worker(rank, world, port, q, bench_cfg=False):
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
     try:
-        torch.cuda.set_device(rank % torch.cuda.device_count())
+        dev = bench.rank_device(rank, torch.cuda.device_count())
+        torch.cuda.set_device(dev)
 
         def gather(obj):
             out = [None] * world
@@ -42,8 +43,11 @@ def _worker(rank, world, port, q, bench_cfg=False):
 
         # run-ahead with type priority, or the launch configuration bench.py times (ready mode,
         # bottom-level priority, 12 slots, group_hold: grouping is off across ranks)
-        rt = vs.Runtime(bench.bench_config(vs, lam=1) if bench_cfg else
-                        vs.vs_config_default(lam=1, slots_per_gpu=2, priority=1))
+        rt = vs.Runtime(bench.bench_config(vs, lam=1, device_base=dev) if bench_cfg else
+                        vs.vs_config_default(lam=1, slots_per_gpu=2, priority=1, device_base=dev))
+        # rank r drives GPU r (bench.rank_device), and creating the runtime left the thread's
+        # current device alone
+        assert rt.vs_gpu_ordinal(0) == dev and torch.cuda.current_device() == dev
         shm = gather("/vsched_test_%d" % os.getpid() if rank == 0 else None)[0]
         if rank == 0:
             rt.vs_dist_init(rank, world, shm)
@@ -79,6 +83,8 @@ def _worker(rank, world, port, q, bench_cfg=False):
                 got, ref = np.tril(got), np.tril(ref)
             err_ch = max(err_ch, oracle.relF(got, ref))
         st = rt.vs_stats()
+        assert torch.cuda.current_device() == dev
+        assert wl.C.device.index == dev and wl.S.device.index == dev
         q.put((rank, err_mm, err_ch, len(own), len(ownc), st.tasks_completed, st.device_tx_bytes, st.tracker, info))
         dist.barrier()
         rt.close()
@@ -113,3 +119,37 @@ def test_two_ranks_sharded_matmul_cholesky(gpu, bench_cfg):
         assert dtx > 0                           # remote tiles were pulled
     for p in procs:
         assert p.exitcode == 0
+
+
+def test_runtime_binds_device_base_and_keeps_current_device(gpu):
+    """vs_config.device_base selects the CUDA device of runtime gpu 0; vs_create / vs_wait_all /
+    vs_destroy leave the caller's current device as it was (one process per GPU, §8(e))."""
+    import torch
+
+    import bench
+    import paper_conf_ipps_planasbal13_b200 as vs
+    ndev = torch.cuda.device_count()
+    for local in range(min(ndev, 8)):
+        dev = bench.rank_device(local, ndev)
+        torch.cuda.set_device(dev)
+        rt = vs.Runtime(vs.vs_config_default(lam=1, slots_per_gpu=2, device_base=dev))
+        assert rt.vs_gpu_ordinal(0) == dev and torch.cuda.current_device() == dev
+        types = rt.vs_register_builtins(vs.VS_F32, 1 << vs.VS_V_SIMT_F32)
+        b = 64
+        T = torch.ones((3, b, b), device="cuda:%d" % dev)
+        ids = [rt.vs_data_register(T[i].data_ptr(), 0, b * b * 4) for i in range(3)]
+        rt.vs_submit(types[vs.VS_T_MATMUL], ids)
+        rt.vs_wait_all()
+        assert torch.cuda.current_device() == dev
+        assert float(T[2, 0, 0]) == 1.0 + b        # C += A B on the rank's own device
+        rt.close()
+    torch.cuda.set_device(0)
+
+
+def test_two_ranks_on_two_gpus_use_their_own_device(gpu):
+    """torchrun-style job with CUDA_VISIBLE_DEVICES unset: rank r's runtime, tiles and kernels are
+    on device r (skipped on a box with one GPU, where the sharded test above shares it)."""
+    import torch
+    if torch.cuda.device_count() < 2:
+        pytest.skip("needs 2 GPUs")
+    test_two_ranks_sharded_matmul_cholesky(gpu, True)
