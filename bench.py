@@ -581,7 +581,11 @@ def main():
             "tensor_pipe_fraction_step": round(frac_step, 4) if world == 1 else None,
             "roofline": roof,
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
-            "dependence_tracker": "device completion words (stream memops)" if st1.tracker == 1 else "cuda events",
+            "dependence_tracker": ("device in-degree counters + CSR successors, ready ring (a3): %d of %d tasks released "
+                                   "on the GPU" % (st1.device_released - st0.device_released,
+                                                   st1.tasks_completed - st0.tasks_completed))
+            if st1.device_released > st0.device_released else
+            "device completion words (stream memops)" if st1.tracker == 1 else "host (completion ring + cuda events)",
             "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "group_tasks": args.group,
                                 "group_hold": args.hold, "group_wait_us": args.group_us,
                                 "mode": args.mode, "cuda_device_max_connections": os.environ.get("CUDA_DEVICE_MAX_CONNECTIONS")},

@@ -164,6 +164,14 @@ typedef struct {
                           stream would otherwise idle); the others keep collecting tasks until
                           group_wait_us.  Fewer, larger launches: the host issues ~1 launch per
                           2.5 tasks instead of ~1 per task in ready mode.  0: launch them all */
+    int device_release; /* 1: device dependence tracker (a3; L400-405): ready mode, one GPU, one
+                          process — at the start of a batch the runtime copies every task's
+                          in-degree and CSR successor list to the GPU; the last CTA of a task's
+                          last kernel (or a one-warp kernel after a user version) decrements
+                          its successors' in-degrees and appends those reaching zero to a
+                          host-mapped ready ring, which the host reads instead of counting
+                          predecessors.  0: the host releases successors.  VS_TRACKER=device /
+                          host overrides */
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,
@@ -277,6 +285,7 @@ typedef struct {
     int64_t host_ns_vevent;   /* host time advancing the virtual clock (run-ahead DES) */
     int64_t host_ns_flush;    /* host time launching pending grouped launches from the loop */
     int64_t host_idle_loops;  /* drive-loop iterations that found nothing to do */
+    int64_t device_released;  /* tasks made ready by the device dependence tracker (a3) */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 

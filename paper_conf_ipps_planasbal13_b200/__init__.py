@@ -41,7 +41,8 @@ class vs_config(Structure):
                 ("lambda_", c_int), ("policy", c_int), ("fixed_version", c_int), ("learning", c_int),
                 ("mode", c_int), ("replay", c_int), ("flush", c_int), ("lookahead", c_int), ("priority", c_int),
                 ("group_ratio_permille", c_int), ("ewma_weight", c_int), ("locality_gbps", c_int),
-                ("queue_depth", c_int), ("group_tasks", c_int), ("group_wait_us", c_int), ("group_hold", c_int)]
+                ("queue_depth", c_int), ("group_tasks", c_int), ("group_wait_us", c_int), ("group_hold", c_int),
+                ("device_release", c_int)]
 
 
 class vs_stats_t(Structure):
@@ -49,7 +50,7 @@ class vs_stats_t(Structure):
         "tasks_submitted", "tasks_completed", "decisions", "input_tx_bytes", "output_tx_bytes", "device_tx_bytes",
         "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns",
         "kernel_launches", "tracker", "forms_built", "host_ns_poll", "host_ns_launch", "host_ns_deps", "host_loops", "host_ns_vevent", "host_ns_flush",
-        "host_idle_loops")]
+        "host_idle_loops", "device_released")]
 
 
 class vs_group_stat_t(Structure):
@@ -280,7 +281,17 @@ class Runtime:
         return out.value
 
     def vs_version_add(self, ttype, name, gpu_mask, fn=None, user=None):
-        cb = VS_LAUNCH_FN(fn) if fn is not None else ctypes.cast(None, VS_LAUNCH_FN)
+        """fn: a C function (a ctypes function of a loaded library, or its address as an int:
+        called by the runtime directly, no Python in the loop), or a Python callable with the
+        vs_launch_fn signature (called through a ctypes trampoline), or None (SIM only)."""
+        if fn is None:
+            cb = ctypes.cast(None, VS_LAUNCH_FN)
+        elif isinstance(fn, int):
+            cb = VS_LAUNCH_FN(fn)
+        elif isinstance(fn, ctypes._CFuncPtr):
+            cb = ctypes.cast(fn, VS_LAUNCH_FN)
+        else:
+            cb = VS_LAUNCH_FN(fn)
         self._keep.append(cb)
         out = c_int32()
         self._ck(lib().vs_version_add(self.h, ttype, name.encode(), gpu_mask, cb, user, ctypes.byref(out)),

@@ -19,6 +19,9 @@
 // A22 -= A21 A21^T (lower GEMM); potrf(A22), down to an NB x NB diagonal block factored
 // in registers (simt_chol.cuh).  Blocked trsm: NB-wide panels solved by trsm_panel,
 // remaining columns updated by the engine's GEMM.
+#include <map>
+#include <mutex>
+#include <tuple>
 #include <type_traits>
 
 #include "dmma_gemm.cuh"
@@ -27,6 +30,7 @@
 #include "simt_gemm.cuh"
 #include "tc_gemm.cuh"
 #include "tc_f16.cuh"
+#include "tc_f16v2.cuh"
 #include "tc_oz.cuh"
 #include "tc_panel.cuh"
 
@@ -201,8 +205,9 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
     if (form == FORM_OZ_ROWS) return oz::make_slices((const double *)src, b, b, b, 1, 128, dst, s);
     if (form == FORM_OZ_ROWS_B) return oz::make_slices((const double *)src, b, b, b, 1, 64, dst, s);
     if (form == FORM_OZ_COLS) return oz::make_slices((const double *)src, b, b, 1, b, 64, dst, s);
-    if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
-    if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
+    const int gr = tcf2::form_group_rows();   // split-form layout of the tc_3xf16 GEMM in use
+    if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s, gr);
+    if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s, gr);
     if (form == FORM_INV_L) {
         // X = I L^{-T} by the substitution kernel of tc_3xtf32 (tc_panel), then the row
         // split form of X^T = inv(L): reading R31 (TRSM of tc_3xf16 multiplies by it)
@@ -210,7 +215,7 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
         count_launch();
         tcf::eye_kernel<<<148, 256, 0, s>>>(X, b);
         if (tc::tc_trsm(b, b, (const float *)src, b, X, b, s)) return -1;
-        return tcf::split_cols(X, b, b, b, dst, s);
+        return tcf::split_cols(X, b, b, b, dst, s, gr);
     }
     return -1;
 }
@@ -231,6 +236,15 @@ int group_ctas(const TaskGroup *g) { return g->g.ctas; }
 // the K-chunk [k0, k0 + kc) of one tc_3xf16 task (kc < 0: all of K)
 static int group_add_chunk(TaskGroup *g, int type, int b, void *const *p, const TaskCtx &ctx, int k0, int kc)
 {
+    if (tcf2::enabled()) {   // persistent CTA-pair kernel (tc_f16v2.cuh)
+        switch (type) {
+        case VS_T_MATMUL: return tcf2::group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, false, false, ctx, false, k0, kc);
+        case VS_T_GEMM_NT: return tcf2::group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, true, false, ctx, false, k0, kc);
+        case VS_T_SYRK: return tcf2::group_add(g->g, b, b, b, p[2], p[2], (float *)p[1], b, true, true, ctx, false, k0, kc);
+        case VS_T_TRSM: return tcf2::group_add(g->g, b, b, b, p[3], p[2], (float *)p[1], b, false, false, ctx, k0 == 0, k0, kc);
+        }
+        return -1;
+    }
     switch (type) {   // p[i] tiles, p[np + i] forms (np = 3 / 2 / 2)
     case VS_T_MATMUL: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, false, false, ctx, false, k0, kc);
     case VS_T_GEMM_NT: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, true, false, ctx, false, k0, kc);
@@ -245,7 +259,10 @@ int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const 
     if (!group_kind(type, version, b)) return -1;
     return group_add_chunk(g, type, b, p, ctx, 0, -1);
 }
-int group_launch(TaskGroup *g, cudaStream_t s) { return tcf::tcf_group_launch(g->g, s); }
+int group_launch(TaskGroup *g, cudaStream_t s)
+{
+    return tcf2::enabled() ? tcf2::group_launch(g->g, s) : tcf::tcf_group_launch(g->g, s);
+}
 
 namespace {
 // oz_i8_f64: p[np + i] holds the slice forms of the in-operands (builtin_operand_form)
@@ -271,6 +288,44 @@ int run_f16(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
     return 0;
 }
 }  // namespace
+
+int builtin_kernel_count(int type, int version, int b)
+{
+    static std::mutex mu;
+    static std::map<std::tuple<int, int, int>, int> cache;
+    if (!builtin_supported(type, version, b)) return -1;
+    std::lock_guard<std::mutex> lock(mu);
+    const auto key = std::make_tuple(type, version, b);
+    auto it = cache.find(key);
+    if (it != cache.end()) return it->second;
+    // capture one launch into a graph (nothing executes; pointers are never dereferenced)
+    cudaStream_t st = nullptr;
+    if (cudaStreamCreateWithFlags(&st, cudaStreamNonBlocking) != cudaSuccess) return -1;
+    void *fake[8];
+    for (int i = 0; i < 8; i++) fake[i] = (void *)(uintptr_t)(0x100000 * (i + 1));
+    int n = -1;
+    const long long c0 = launch_counter().load();
+    if (cudaStreamBeginCapture(st, cudaStreamCaptureModeThreadLocal) == cudaSuccess) {
+        const int r = launch_builtin(type, version, b, fake, (int *)fake[7], st);
+        cudaGraph_t g = nullptr;
+        const bool ok = cudaStreamEndCapture(st, &g) == cudaSuccess && r == 0;
+        if (ok) n = (int)(launch_counter().load() - c0);
+        if (g) cudaGraphDestroy(g);
+    }
+    launch_counter().fetch_sub(launch_counter().load() - c0);   // captured, never launched
+    cudaGetLastError();
+    cudaStreamDestroy(st);
+    if (n >= 0) cache[key] = n;
+    return n;
+}
+
+int launch_release(const TaskCtx &ctx, cudaStream_t s)
+{
+    if (!ctx.trk) return 0;
+    count_launch();
+    release_kernel<<<1, 32, 0, s>>>(ctx);
+    return cudaGetLastError() == cudaSuccess ? 0 : -1;
+}
 
 int launch_builtin(int type, int version, int b, void *const *p, int *info, cudaStream_t s, const TaskCtx &ctx)
 {

@@ -105,7 +105,8 @@ inline void dmma_gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, 
     if (M <= 0 || N <= 0) return;
     dim3 grid((N + 63) / 64, (M + 63) / 64);
     count_launch();
-    dmma_gemm_kernel<Tin, NT, NEG, LOWER><<<grid, 128, 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc, ctx);
+    auto kern = dmma_gemm_kernel<Tin, NT, NEG, LOWER>;
+    kern<<<grid, 128, 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc, ctx_for(ctx, kern, 128, 0));
 }
 
 }  // namespace vsk

@@ -16,6 +16,21 @@ inline std::atomic<long long> &launch_counter()
 }
 inline void count_launch() { launch_counter().fetch_add(1, std::memory_order_relaxed); }
 
+// Device dependence tracker (a3): in-degrees and CSR successor lists of
+// the tasks of one drive, in device memory of the runtime's GPU, built by the runtime at the
+// start of the drive.  Task index = task id - first id of the batch.  The last CTA of a task's
+// last kernel decrements the in-degree of each successor; a successor whose count reaches zero
+// is appended to the host-mapped ready ring (entry = epoch << 32 | index + 1), which the host
+// reads instead of counting predecessors itself.
+struct DevTracker {
+    int *indeg = nullptr;                    // [T] predecessors not yet complete
+    const int *succ_off = nullptr;           // [T + 1]
+    const int *succ = nullptr;               // [E]
+    unsigned long long *rdy_ctr = nullptr;   // device counter of ready-ring entries
+    unsigned long long *rdy_ring = nullptr;  // host-mapped ring (kRingCap entries, 0 = empty)
+    unsigned long long epoch = 0;            // drive number (stale entries are ignored)
+};
+
 // Per-task execution record passed to every kernel of a built-in version (task_ctx.cuh).
 // slot: device memory {start_min, end_max, ticket}; host: host-mapped {start, end,
 // kernels completed, pad}.
@@ -24,12 +39,17 @@ struct TaskCtx {
     unsigned long long *slot = nullptr;   // device {~start min, end max, CTA ticket, CTA busy sum, longest CTA, -}
     unsigned long long *host = nullptr;   // host-mapped {~start, end, kernels done, exec time}
     unsigned int ncta = 0;   // CTAs of the task in the launch (0: the whole grid)
-    unsigned int nsm = 0;    // SMs of the device (CTAs that can run at once, 1 per SM)
+    unsigned int nsm = 0;    // SMs of the device
+    unsigned int occ = 0;    // resident CTAs per SM of the kernel (occupancy; 0 = 1), set per launch
     // completion ring (host-mapped): the last CTA of every kernel of the task appends `tag`
     // at ring[atomicAdd(ring_ctr) % kRingCap], so the host reads completions in O(completed)
     unsigned long long *ring_ctr = nullptr;   // device counter of appended entries
     unsigned long long *ring = nullptr;       // host-mapped entries (0 = empty)
     unsigned long long tag = 0;               // task id + 1
+    // device dependence release (a3): null = the host releases successors
+    const DevTracker *trk = nullptr;
+    int tidx = 0;              // task index in trk
+    unsigned int nkern = 0;    // kernels of the task: the last one releases
 };
 constexpr unsigned long long kRingCap = 1ull << 16;
 
@@ -37,6 +57,11 @@ constexpr unsigned long long kRingCap = 1ull << 16;
 // Returns 0 on success, -1 for an unsupported (type, version, b).
 int launch_builtin(int type, int version, int b, void *const *p, int *dinfo, cudaStream_t s,
                    const TaskCtx &ctx = TaskCtx());
+// Kernels launch_builtin enqueues for (type, version, b) (counted once by capturing a launch
+// into a CUDA graph; cached), -1 if unsupported.
+int builtin_kernel_count(int type, int version, int b);
+// One-warp kernel doing only the dependence release of ctx (after a user version's work).
+int launch_release(const TaskCtx &ctx, cudaStream_t s);
 bool builtin_supported(int type, int version, int b);
 // Element size in bytes for a version (4 for f32-io versions, 8 for f64).
 int builtin_elem_bytes(int version);

@@ -124,7 +124,8 @@ inline void trsm_panel(const Tin *L, int ldl, Tin *X, int ldx, int rows, cudaStr
 {
     if (rows <= 0) return;
     count_launch();
-    trsm_panel_kernel<Tin, Tacc, NB><<<(rows + 63) / 64, 64, 0, s>>>(L, ldl, X, ldx, rows, ctx);
+    auto kern = trsm_panel_kernel<Tin, Tacc, NB>;
+    kern<<<(rows + 63) / 64, 64, 0, s>>>(L, ldl, X, ldx, rows, ctx_for(ctx, kern, 64, 0));
 }
 
 }  // namespace vsk

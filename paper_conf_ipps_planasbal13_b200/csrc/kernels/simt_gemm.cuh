@@ -156,8 +156,9 @@ inline void simt_gemm(int M, int N, int K, const Tin *A, int lda, const Tin *B, 
     constexpr int BM = WIDE ? 128 : 64, BN = WIDE ? 128 : 64, BK = 16, TM = WIDE ? 8 : 4, TN = WIDE ? 8 : 4;
     dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
     count_launch();
-    simt_gemm_kernel<Tin, Tacc, BM, BN, BK, TM, TN, NT, NEG, LOWER>
-        <<<grid, (BM / TM) * (BN / TN), 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc, ctx);
+    auto kern = simt_gemm_kernel<Tin, Tacc, BM, BN, BK, TM, TN, NT, NEG, LOWER>;
+    constexpr int threads = (BM / TM) * (BN / TN);
+    kern<<<grid, threads, 0, s>>>(M, N, K, A, lda, B, ldb, C, ldc, ctx_for(ctx, kern, threads, 0));
 }
 
 }  // namespace vsk

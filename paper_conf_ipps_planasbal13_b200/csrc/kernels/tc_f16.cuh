@@ -100,14 +100,15 @@ __host__ __device__ inline size_t split_bytes(int R, int K)
     return Rp * (size_t)K * 4 + Rp * 8;
 }
 // byte offset of the 16-byte chunk holding elements (r, 8c .. 8c+7) of the big part; the
-// small part of the same chunk is SPLIT_HALF bytes further (big and small of one 256-row
-// group are adjacent, so one 32 KB bulk copy moves both)
+// small part of the same chunk is GR * 64 bytes further (big and small of one GR-row group
+// are adjacent, so one bulk copy moves both: 32 KB for GR = 256, the CTA tile of
+// tcf_gemm_kernel; 16 KB for GR = 128, one CTA's half of the CTA-pair tile of tc_f16v2.cuh)
 constexpr int SPLIT_HALF = 256 * 64;
+template <int GR = 256>
 __host__ __device__ inline size_t split_chunk_off(int Rp, int r, int c)
 {
     const int kb = c >> 2, kc = c & 3;
-    return (size_t)kb * Rp * 128 + (size_t)(r >> 8) * (2 * SPLIT_HALF) + (size_t)(r & 255) * 64 +
-           ((kc ^ ((r >> 1) & 3)) << 4);
+    return (size_t)kb * Rp * 128 + (size_t)(r / GR) * (2 * GR * 64) + (size_t)(r % GR) * 64 + ((kc ^ ((r >> 1) & 3)) << 4);
 }
 
 // Row scale exponent: max * 2^e in [2^14, 2^15).
@@ -140,6 +141,7 @@ __device__ __forceinline__ void split8(const float (&v)[8], float sc, uint4 &big
 }
 
 // Row form of an R x K row-major fp32 matrix (ld): one warp per (padded) row.
+template <int GR>
 __global__ void __launch_bounds__(256) split_rows_kernel(const float *__restrict__ X, int R, int K, int ld,
                                                          uint8_t *__restrict__ out)
 {
@@ -160,7 +162,7 @@ __global__ void __launch_bounds__(256) split_rows_kernel(const float *__restrict
     }
     const int e = row_exponent(m);
     const float sc = ldexpf(1.f, e);
-    const size_t half = SPLIT_HALF;
+    const size_t half = (size_t)GR * 64;
     for (int k = 8 * lane; k < K; k += 256) {
         float v[8] = {0.f, 0.f, 0.f, 0.f, 0.f, 0.f, 0.f, 0.f};
         if (r < R) {
@@ -170,7 +172,7 @@ __global__ void __launch_bounds__(256) split_rows_kernel(const float *__restrict
         }
         uint4 big, small;
         split8(v, sc, big, small);
-        const size_t off = split_chunk_off(Rp, r, k >> 3);
+        const size_t off = split_chunk_off<GR>(Rp, r, k >> 3);
         *reinterpret_cast<uint4 *>(out + off) = big;
         *reinterpret_cast<uint4 *>(out + off + half) = small;
     }
@@ -203,6 +205,7 @@ __global__ void __launch_bounds__(256) split_colmax_kernel(const float *__restri
     }
 }
 
+template <int GR>
 __global__ void __launch_bounds__(256) split_cols_kernel(const float *__restrict__ X, int K, int R, int ld,
                                                          uint8_t *__restrict__ out)
 {
@@ -226,9 +229,9 @@ __global__ void __launch_bounds__(256) split_cols_kernel(const float *__restrict
         for (int i = 0; i < 8; i++) v[i] = tile[kc * 8 + i][rr];
         uint4 big, small;
         split8(v, ldexpf(1.f, e), big, small);
-        const size_t off = split_chunk_off(Rp, r0 + rr, (k0 >> 3) + kc);
+        const size_t off = split_chunk_off<GR>(Rp, r0 + rr, (k0 >> 3) + kc);
         *reinterpret_cast<uint4 *>(out + off) = big;
-        *reinterpret_cast<uint4 *>(out + off + SPLIT_HALF) = small;
+        *reinterpret_cast<uint4 *>(out + off + (size_t)GR * 64) = small;
     }
 }
 
@@ -554,16 +557,19 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
 
 // ---------------------------------------------------------------- host launchers
 // Split forms: X is R x K row-major (ld) -> row form; X is K x R row-major -> row form of X^T.
-inline int split_rows(const float *X, int R, int K, int ld, void *out, cudaStream_t s)
+// gr: row group of the layout (256: tcf_gemm_kernel, 128: the CTA-pair kernel of tc_f16v2.cuh)
+inline int split_rows(const float *X, int R, int K, int ld, void *out, cudaStream_t s, int gr = 256)
 {
-    if (R <= 0 || K <= 0 || K % 32 || ld % 4) return -1;
+    if (R <= 0 || K <= 0 || K % 32 || ld % 4 || (gr != 256 && gr != 128)) return -1;
     const int Rp = split_rows_padded(R);
     count_launch();
-    split_rows_kernel<<<(Rp + 7) / 8, 256, 0, s>>>(X, R, K, ld, (uint8_t *)out);
+    if (gr == 256) split_rows_kernel<256><<<(Rp + 7) / 8, 256, 0, s>>>(X, R, K, ld, (uint8_t *)out);
+    else split_rows_kernel<128><<<(Rp + 7) / 8, 256, 0, s>>>(X, R, K, ld, (uint8_t *)out);
     return 0;
 }
-inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStream_t s)
+inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStream_t s, int gr = 256)
 {
+    if (gr != 256 && gr != 128) return -1;
     if (R <= 0 || K <= 0 || K % 32) return -1;
     const int Rp = split_rows_padded(R);
     if (cudaMemsetAsync((uint8_t *)out + (size_t)Rp * K * 4 + (size_t)Rp * 4, 0, (size_t)Rp * 4, s) != cudaSuccess)
@@ -571,7 +577,8 @@ inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStrea
     count_launch();
     split_colmax_kernel<<<dim3(Rp / 32, (K + 127) / 128), 256, 0, s>>>(X, K, R, ld, (uint8_t *)out);
     count_launch();
-    split_cols_kernel<<<dim3(Rp / 32, (K + 63) / 64), 256, 0, s>>>(X, K, R, ld, (uint8_t *)out);
+    if (gr == 256) split_cols_kernel<256><<<dim3(Rp / 32, (K + 63) / 64), 256, 0, s>>>(X, K, R, ld, (uint8_t *)out);
+    else split_cols_kernel<128><<<dim3(Rp / 32, (K + 63) / 64), 256, 0, s>>>(X, K, R, ld, (uint8_t *)out);
     return 0;
 }
 

@@ -420,11 +420,12 @@ inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B,
     // 2.9e-5 at 4096).  K is therefore cut into chunks of at most kKChunk, one launch each; every
     // launch adds its chunk to C in fp32 round-to-nearest (the C_in path), which keeps every K at
     // the K = 1024 error (fp32-class gate, BASELINE north star)
+    const TaskCtx c = ctx_for(ctx, kern, NTHREADS, smem);
     for (int k0 = 0; k0 < K; k0 += kKChunk) {
         const int kc = K - k0 < kKChunk ? K - k0 : kKChunk;
         count_launch();
         kern<<<grid, NTHREADS, smem, s>>>(M, N, kc, A + k0, lda, B + (NT ? (int64_t)k0 : (int64_t)k0 * ldb), ldb, C, ldc,
-                                          ctx);
+                                          c);
     }
     return 0;
 }

@@ -362,7 +362,7 @@ inline int oz_gemm(int M, int N, int K, const void *Af, const void *Bf, double *
         attr[dev & 63] = true;
     }
     const dim3 grid((M + BM - 1) / BM, N / BN);
-    TaskCtx c = ctx;
+    TaskCtx c = ctx_for(ctx, oz_gemm_kernel<NEG, LOWER, GB>, NTHREADS, SMEM);
     c.ncta = grid.x * grid.y;
     count_launch();
     oz_gemm_kernel<NEG, LOWER, GB><<<grid, NTHREADS, SMEM, s>>>(M, N, K, (const uint8_t *)Af, (const uint8_t *)Bf, C, ldc, c);

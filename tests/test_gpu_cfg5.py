@@ -21,11 +21,23 @@ pytestmark = pytest.mark.gpu
 sys.path.insert(0, os.path.join(os.path.dirname(os.path.dirname(os.path.abspath(__file__))), "tools"))
 
 
+_GT = {}
+
+
+def _ground_truth(sw, b):
+    """Isolated timing of every version (median of back-to-back launches, nothing co-running):
+    the independent reference the scheduler's picks are judged against."""
+    if b not in _GT:
+        _GT[b] = sw.ground_truth(b, sw.VERSIONS, runs=30)
+    return _GT[b]
+
+
 @pytest.mark.parametrize("lam", [1, 2])
 def test_cfg5_interleaved_convergence(gpu, lam):
     import sweep_cfg5 as sw
     import torch
-    sizes = [128, 256, 512]
+    sizes = [128, 256, 512, 1024]
+    gt = {b: _ground_truth(sw, b) for b in sizes}
     log, groups, task_b, keep = sw.run_sweep_once(lam, sizes, sw.VERSIONS, slots=4)
     V = len(sw.VERSIONS)
     assert len(log) == len(sizes) * 64
@@ -35,16 +47,25 @@ def test_cfg5_interleaved_convergence(gpu, lam):
         recs = [r for r in log if task_b[r[0]] == b]
         learn = [r[1] for r in recs[:V * lam]]
         assert sorted(learn) == sorted(list(range(V)) * lam)
-        # means keep learning in the reliable phase (a14), so a near-tie may switch the pick
-        # mid-run: every pick is a version whose final mean is near the fastest, most are it
-        means = np.array(g["mean_ns"], dtype=np.float64)
-        fastest = int(np.argmin(means))
+        # judged against the isolated ground truth, not the scheduler's own means: every
+        # reliable pick is a version within 25 % of the truly fastest (near-ties may alternate,
+        # since means keep learning, a14), and a clear winner takes most picks
+        t = [gt[b][v] for v in sw.VERSIONS]
+        fastest = int(np.argmin(t))
         post = [r[1] for r in recs[V * lam:]]
-        assert all(means[v] <= 1.5 * means[fastest] for v in post), (b, g)
-        second = min(means[v] for v in range(V) if v != fastest)
-        if second >= 1.2 * means[fastest]:   # a clear winner (not a near-tie) takes most picks
-            assert sum(v == fastest for v in post) >= len(post) // 2, (b, g)
-        if b > 256:
+        assert all(t[v] <= 1.25 * t[fastest] for v in post), (b, t, g)
+        second = min(t[v] for v in range(V) if v != fastest)
+        if second >= 1.2 * t[fastest]:
+            assert sum(v == fastest for v in post) >= len(post) // 2, (b, t, g)
+        # the learned means (R17, recorded under co-running) order the versions as the isolated
+        # timings do wherever they differ by more than 2x, and stay within a factor 2 of them
+        means = np.array(g["mean_ns"], dtype=np.float64) / 1e3
+        for v in range(V):
+            assert 0.5 <= means[v] / t[v] <= 2.0, (b, v, means, t)
+            for u in range(V):
+                if t[u] > 2 * t[v]:
+                    assert means[u] > means[v], (b, u, v, means, t)
+        if b > 512:
             continue
         # parity of the result (C0 = 0, A = u(100+lam), B = u(1100+lam), N = 4b)
         n = 4 * b

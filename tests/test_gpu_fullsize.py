@@ -40,7 +40,15 @@ def test_fullsize_bench_configuration(gpu):
     lhs = Afull.astype(np.float64) @ (Bfull.astype(np.float64) @ x)
     assert np.linalg.norm(lhs - C @ x) / np.linalg.norm(lhs) <= 1e-5
     del C, Afull, Bfull
-    # ---- Cholesky: leading 2048 block vs oracle; residual on the full matrix
+    # ---- Cholesky: leading 8192 block vs oracle at the fp32-class gate; residual on the full
+    # matrix.  L[:k, :k] = chol(A[:k, :k]) exactly (the leading block of a Cholesky factor is the
+    # factor of the leading block), and at b = 1024 the block holds tiles produced by every task
+    # type of the bench: 8 potrf, 28 trsm, 28 syrk and 56 GEMM_NT (the type with 91 % of the
+    # flops), on the versions and grouped launches the bench's scheduler chose.  At this size a
+    # 1xTF32 update measured strict-lower relF ~4e-5, so the 1e-5 gate on the
+    # strict lower triangle (R23) catches it; the whole-matrix residual below is the P3 bound
+    # ||A x - L L^T x|| <= 4 N u ||A x||, a sanity bound that holds for any backward-stable fp32
+    # factorisation, not a parity gate.
     Nc, bc = bench.CH_N, bench.CH_B
     ntc = Nc // bc
 
@@ -54,7 +62,7 @@ def test_fullsize_bench_configuration(gpu):
                 k += 1
         return out
     L = np.tril(full(wl.S))
-    k = 2048
+    k = 8192
     r = np.arange(k, dtype=np.uint64)[:, None]
     c = np.arange(k, dtype=np.uint64)[None, :]
     S = vsgen.uniform_idx(bench.SEED_CH, np.maximum(r, c) * np.uint64(Nc) + np.minimum(r, c))
@@ -62,8 +70,10 @@ def test_fullsize_bench_configuration(gpu):
     Lk, info = oracle.cholesky(S.astype(np.float32))
     assert info == 0
     lo, slo = np.tril_indices(k), np.tril_indices(k, -1)
-    assert oracle.relF(L[:k, :k][lo], Lk[lo]) <= 1e-5
-    assert oracle.relF(L[:k, :k][slo], Lk[slo]) <= 1e-5
+    e_lo, e_slo = oracle.relF(L[:k, :k][lo], Lk[lo]), oracle.relF(L[:k, :k][slo], Lk[slo])
+    print("fullsize cholesky leading %d block: relF tril %.3e strict-lower %.3e" % (k, e_lo, e_slo))
+    assert e_lo <= 1e-5
+    assert e_slo <= 1e-5
     A = full(wl.S0)
     A = np.tril(A) + np.tril(A, -1).T
     x = rng.standard_normal(Nc)

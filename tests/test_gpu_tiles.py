@@ -15,7 +15,7 @@ F64_VERSIONS = [vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64]
 # tc_3xf16 and oz_i8_f64: gemm-type tasks only (tc_3xf16 also TRSM)
 GEMM_VERSIONS = F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS + [vs.VS_V_OZ_I8_F64]
 FP64_STORAGE = (vs.VS_V_DFMA_F64, vs.VS_V_DMMA_F64, vs.VS_V_OZ_I8_F64)
-SIZES = [64, 128, 192, 320, 512]
+SIZES = [64, 128, 192, 320, 512, 1024]   # 1024: the bench's tile size
 
 
 def _torch():
@@ -182,7 +182,7 @@ def test_oz_i8_f64_row_scales_and_componentwise_bound(gpu, ttype):
 
 # ------------------------------------------------------------------ trsm / potrf
 @pytest.mark.parametrize("version", F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS)
-@pytest.mark.parametrize("b", [64, 128, 192, 512])
+@pytest.mark.parametrize("b", [64, 128, 192, 512, 1024])
 def test_trsm_tile(gpu, version, b):
     dt = _dt(version)
     Lfull, _ = oracle.cholesky(vsgen.spd(500 + b, b, np.float64))
@@ -193,7 +193,7 @@ def test_trsm_tile(gpu, version, b):
 
 
 @pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
-@pytest.mark.parametrize("b", [64, 128, 192, 512])
+@pytest.mark.parametrize("b", [64, 128, 192, 512, 1024])
 def test_potrf_tile(gpu, version, b):
     torch = _torch()
     dt = _dt(version)
@@ -207,7 +207,7 @@ def test_potrf_tile(gpu, version, b):
     lo = np.tril_indices(b)
     slo = np.tril_indices(b, -1)
     assert oracle.relF(L[lo], ref[lo]) <= _gate(version)
-    assert oracle.relF(L[slo], ref[slo]) <= 5 * _gate(version)     # R23 strict-lower gate
+    assert oracle.relF(L[slo], ref[slo]) <= _gate(version)         # R23 strict-lower gate
     assert np.all(L[np.triu_indices(b, 1)] == 777.0)                  # R7
 
 

@@ -139,6 +139,9 @@ def analyse(lam, log, groups, task_b, sizes, versions, gt):
             "regret_us": round(regret, 2),
             "gt_us": {vs.VERSION_NAMES[v]: round(t, 2) for v, t in gt[b].items()},
             "mean_us": {g["versions"][i]: round(m / 1e3, 2) for i, m in enumerate(g["mean_ns"])},
+            # learned mean (R17, device-recorded under co-running) / isolated ground truth
+            "mean_over_gt": {g["versions"][i]: round(m / 1e3 / gt[b][versions[i]], 3)
+                             for i, m in enumerate(g["mean_ns"]) if m > 0},
             "n": g["n"]})
     return res
 
@@ -168,6 +171,8 @@ def main():
         "groups_picking_fastest": sum(r["picks_fastest"] for r in allres), "groups": len(allres),
         "groups_picking_within_5pct": sum(r["picks_within_5pct"] for r in allres),
         "mean_frac_fastest": round(sum(r["frac_fastest"] for r in allres) / len(allres), 4),
+        "mean_over_gt_range": [min(x for r in allres for x in r["mean_over_gt"].values()),
+                               max(x for r in allres for x in r["mean_over_gt"].values())],
         "total_regret_us": round(sum(r["regret_us"] for r in allres), 1)}
     print(json.dumps(summary))
     if a.out:
