@@ -110,14 +110,18 @@ class Workload:
     one rank) keeps the tiles in pinned host memory and lets the runtime move them."""
 
     def __init__(self, rt, mm_n=MM_N, mm_b=MM_B, ch_n=CH_N, ch_b=CH_B, host=False, rank=0, nranks=1, gather=None,
-                 mask=F32_VERSIONS_MASK, with_mm=True, with_ch=True):
+                 mask=F32_VERSIONS_MASK, with_mm=True, with_ch=True, f64=False, seeds=(SEED_MM, SEED_CH)):
         import torch
         import paper_conf_ipps_planasbal13_b200 as vs
         self.torch, self.vs, self.rt = torch, vs, rt
         self.mm_n, self.mm_b, self.ch_n, self.ch_b, self.host = mm_n, mm_b, ch_n, ch_b, host
         self.rank, self.nranks = rank, nranks
         self.with_mm, self.with_ch = with_mm, with_ch
-        self.types = rt.vs_register_builtins(vs.VS_F32, mask)
+        self.vdt = vs.VS_F64 if f64 else vs.VS_F32
+        self.tdt = torch.float64 if f64 else torch.float32
+        self.esize = 8 if f64 else 4
+        seed_mm, seed_ch = seeds
+        self.types = rt.vs_register_builtins(self.vdt, mask)
         self.flops = 0.0
         self.ids = []            # every registered datum (for invalidation)
         self.opened = []         # IPC bases to close
@@ -126,9 +130,9 @@ class Workload:
             self.mm_nt = nt
             all_t = [(i, j) for i in range(nt) for j in range(nt)]
             self.A, self.ia = self._matrix("A", all_t, mm_b, mm_n, lambda T, k, i, j: vs.vs_gen_tile(
-                SEED_MM, mm_n, mm_n, vs.VS_F32, mm_b, i, j, 0, T[k].data_ptr()), gather)
+                seed_mm, mm_n, mm_n, self.vdt, mm_b, i, j, 0, T[k].data_ptr()), gather)
             self.B, self.ib = self._matrix("B", all_t, mm_b, mm_n, lambda T, k, i, j: vs.vs_gen_tile(
-                SEED_MM + 1000, mm_n, mm_n, vs.VS_F32, mm_b, i, j, 0, T[k].data_ptr()), gather)
+                seed_mm + 1000, mm_n, mm_n, self.vdt, mm_b, i, j, 0, T[k].data_ptr()), gather)
             self.C, self.ic = self._matrix("C", all_t, mm_b, mm_n, None, gather)
             self.flops += MM_FLOPS(mm_n)
         if with_ch:
@@ -136,7 +140,7 @@ class Workload:
             self.ch_nt = nt
             low = [(i, j) for i in range(nt) for j in range(i + 1)]
             self.S, idl = self._matrix("S", low, ch_b, ch_n, lambda T, k, i, j: vs.vs_gen_tile(
-                SEED_CH, ch_n, ch_n, vs.VS_F32, ch_b, i, j, 1, T[k].data_ptr()), gather)
+                seed_ch, ch_n, ch_n, self.vdt, ch_b, i, j, 1, T[k].data_ptr()), gather)
             self.S0 = self.S.clone()
             self.iS = {i * nt + j: d for (i, j), d in zip(low, idl)}
             self.flops += CH_FLOPS(ch_n)
@@ -146,13 +150,13 @@ class Workload:
         """Allocate this rank's tiles of one matrix (one buffer), register every tile."""
         torch, vs, rt = self.torch, self.vs, self.rt
         own = [t for t in tiles if tile_owner(t[0], t[1], self.nranks) == self.rank]
-        T = torch.zeros((max(1, len(own)), b, b), dtype=torch.float32, device="cuda")
+        T = torch.zeros((max(1, len(own)), b, b), dtype=self.tdt, device="cuda")
         if gen is not None:
             for k, (i, j) in enumerate(own):
                 gen(T, k, i, j)
         if self.host:
             T = T.cpu().pin_memory()
-        nbytes = b * b * 4
+        nbytes = b * b * self.esize
         dev = -1 if self.host else 0
         ids = {}
         for k, t in enumerate(own):
@@ -339,6 +343,66 @@ def config_json(args, world, mm_n=MM_N, mm_b=MM_B, ch_n=CH_N, ch_b=CH_B, with_mm
             "l2": "inputs larger than L2 (4 GiB + 4 GiB)", "regime": "warm (tables learned in warm-up)"}
 
 
+# ----------------------------------------------------------------------------- per-config record
+# (name, matmul (N, b) or None, Cholesky (N, b) or None, fp64?, version mask, what it is)
+V = lambda *vv: sum(1 << v for v in vv)   # noqa: E731
+CONFIGS = [
+    ("cfg1_matmul_1024_b256", (1024, 256), None, False, V(0, 1),
+     "BASELINE cfg1: tiled matmul N=1024 fp32, 256x256 tiles, versions simt_f32/tc_3xtf32"),
+    ("cfg2_cholesky_4096_b512", None, (4096, 512), False, V(0, 1, 2),
+     "BASELINE cfg2: tiled Cholesky N=4096 SPD fp32, 512x512 tiles, versions simt_f32/tc_3xtf32/f64in_f32io"),
+    ("cfg3_matmul_16384_b1024", (16384, 1024), None, False, F32_VERSIONS_MASK,
+     "BASELINE cfg3 alone: tiled matmul N=16384 fp32, 1024x1024 tiles, all f32 versions"),
+    ("cfg4_cholesky_32768_b1024", None, (32768, 1024), False, F32_VERSIONS_MASK,
+     "BASELINE cfg4 alone: tiled Cholesky N=32768 SPD fp32, 1024x1024 tiles, all f32 versions"),
+    ("paper_fp64_matmul_16384_b1024", (16384, 1024), None, True, V(3, 4, 6),
+     "paper-shaped matmul (L611-612, reading R3): fp64 N=16384, 1024x1024 tiles, versions dfma_f64/dmma_f64/"
+     "oz_i8_f64 (the tcgen05 kind::i8 Ozaki version)"),
+    ("paper_cholesky_32768_b2048", None, (32768, 2048), False, F32_VERSIONS_MASK,
+     "paper-shaped Cholesky (L700-703, reading R4): fp32 N=32768, 2048x2048 tiles (816 tasks)"),
+]
+
+
+def measure_config(args, vs, torch, name, mm, ch, f64, mask, what, steps=3, warmup=2):
+    """One config on its own runtime (the bench's launch configuration), warm: `warmup` untimed
+    steps (learning happens in the first), then `steps` steps timed with CUDA events."""
+    cfg = bench_config(vs, lam=args.lam, slots_per_gpu=args.slots, priority=args.priority, queue_depth=args.qdepth,
+                       group_tasks=args.group, group_hold=args.hold, group_wait_us=args.group_us)
+    rt = vs.Runtime(cfg)
+    kw = dict(with_mm=mm is not None, with_ch=ch is not None, mask=mask, f64=f64)
+    wl = Workload(rt, mm[0] if mm else MM_N, mm[1] if mm else MM_B, ch[0] if ch else CH_N, ch[1] if ch else CH_B, **kw)
+    for _ in range(warmup):
+        wl.step()
+    st0 = rt.vs_stats()
+    rt.vs_decision_log_clear()
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record()
+    for _ in range(steps):
+        wl.step()
+    e1.record()
+    torch.cuda.synchronize()
+    ms = e0.elapsed_time(e1) / steps
+    st1 = rt.vs_stats()
+    groups = rt.vs_group_stats()
+    picks = {}
+    for r in rt.vs_decision_log():
+        g = next(x for x in groups if x["type"] == r[7])
+        k = "%s/%s" % (g["type_name"], g["versions"][r[1]])
+        picks[k] = picks.get(k, 0) + 1
+    tasks = (st1.tasks_completed - st0.tasks_completed) // steps
+    out = {"what": what, "value": round(wl.flops / (ms * 1e-3) / 1e9, 1), "unit": "GFLOP/s",
+           "ms_per_step": round(ms, 3), "steps": steps, "warmup": warmup, "tasks_per_step": int(tasks),
+           "us_per_task_step": round(1e3 * ms / max(1, tasks), 2), "dtype": "f64" if f64 else "f32",
+           "decisions_per_step": {k: v // steps for k, v in sorted(picks.items())},
+           "learned_mean_us": {"%s/%s" % (g["type_name"], v): round(m / 1e3, 1) for g in groups
+                               for v, m in zip(g["versions"], g["mean_ns"]) if m}}
+    rt.close()
+    del wl
+    torch.cuda.empty_cache()
+    return out
+
+
 # ----------------------------------------------------------------------------- reference arm
 _CPU = {}
 
@@ -432,6 +496,8 @@ def main():
     ap.add_argument("--table-dump", default="", help="write the learned TaskVersionSets after warm-up")
     ap.add_argument("--table-load", default="", help="warm start from a table (NEXT-2 hints)")
     ap.add_argument("--replay", action="store_true", help="decisions from the loaded table (profiling runs)")
+    ap.add_argument("--no-configs", action="store_true", help="skip the per-config record (cfg1..cfg4 alone, "
+                    "paper-shaped fp64 matmul and b=2048 Cholesky) measured after the timed region")
     args = ap.parse_args()
     rank = int(os.environ.get("RANK", "0"))
     world = int(os.environ.get("WORLD_SIZE", "1"))
@@ -559,6 +625,16 @@ def main():
         rt2.close()
         del wl2
 
+    # ---- per-config record (after the timed region and the e2e leg; one GPU)
+    configs = None
+    if world == 1 and not args.no_configs and not args.small and args.only == "both":
+        configs = {}
+        for (name, mm, ch, f64, mask, what) in CONFIGS:
+            try:
+                configs[name] = measure_config(args, vs, torch, name, mm, ch, f64, mask, what)
+            except Exception as ex:   # a failing extra record must not lose the main line
+                configs[name] = {"what": what, "error": repr(ex)[:300]}
+
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu:
         s = cpu_sample()
@@ -581,6 +657,7 @@ def main():
             "tensor_pipe_fraction_step": round(frac_step, 4) if world == 1 else None,
             "roofline": roof,
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches), "clocks": clocks,
+            "configs": configs,
             "dependence_tracker": ("device in-degree counters + CSR successors, ready ring (a3): %d of %d tasks released "
                                    "on the GPU" % (st1.device_released - st0.device_released,
                                                    st1.tasks_completed - st0.tasks_completed))

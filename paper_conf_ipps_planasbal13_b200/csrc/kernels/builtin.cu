@@ -30,7 +30,6 @@
 #include "simt_gemm.cuh"
 #include "tc_gemm.cuh"
 #include "tc_f16.cuh"
-#include "tc_f16v2.cuh"
 #include "tc_oz.cuh"
 #include "tc_panel.cuh"
 
@@ -205,9 +204,8 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
     if (form == FORM_OZ_ROWS) return oz::make_slices((const double *)src, b, b, b, 1, 128, dst, s);
     if (form == FORM_OZ_ROWS_B) return oz::make_slices((const double *)src, b, b, b, 1, 64, dst, s);
     if (form == FORM_OZ_COLS) return oz::make_slices((const double *)src, b, b, 1, b, 64, dst, s);
-    const int gr = tcf2::form_group_rows();   // split-form layout of the tc_3xf16 GEMM in use
-    if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s, gr);
-    if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s, gr);
+    if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
+    if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
     if (form == FORM_INV_L) {
         // X = I L^{-T} by the substitution kernel of tc_3xtf32 (tc_panel), then the row
         // split form of X^T = inv(L): reading R31 (TRSM of tc_3xf16 multiplies by it)
@@ -215,7 +213,7 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
         count_launch();
         tcf::eye_kernel<<<148, 256, 0, s>>>(X, b);
         if (tc::tc_trsm(b, b, (const float *)src, b, X, b, s)) return -1;
-        return tcf::split_cols(X, b, b, b, dst, s, gr);
+        return tcf::split_cols(X, b, b, b, dst, s);
     }
     return -1;
 }
@@ -236,15 +234,6 @@ int group_ctas(const TaskGroup *g) { return g->g.ctas; }
 // the K-chunk [k0, k0 + kc) of one tc_3xf16 task (kc < 0: all of K)
 static int group_add_chunk(TaskGroup *g, int type, int b, void *const *p, const TaskCtx &ctx, int k0, int kc)
 {
-    if (tcf2::enabled()) {   // persistent CTA-pair kernel (tc_f16v2.cuh)
-        switch (type) {
-        case VS_T_MATMUL: return tcf2::group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, false, false, ctx, false, k0, kc);
-        case VS_T_GEMM_NT: return tcf2::group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, true, false, ctx, false, k0, kc);
-        case VS_T_SYRK: return tcf2::group_add(g->g, b, b, b, p[2], p[2], (float *)p[1], b, true, true, ctx, false, k0, kc);
-        case VS_T_TRSM: return tcf2::group_add(g->g, b, b, b, p[3], p[2], (float *)p[1], b, false, false, ctx, k0 == 0, k0, kc);
-        }
-        return -1;
-    }
     switch (type) {   // p[i] tiles, p[np + i] forms (np = 3 / 2 / 2)
     case VS_T_MATMUL: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, false, false, ctx, false, k0, kc);
     case VS_T_GEMM_NT: return tcf::tcf_group_add(g->g, b, b, b, p[3], p[4], (float *)p[2], b, true, false, ctx, false, k0, kc);
@@ -259,10 +248,7 @@ int group_add(TaskGroup *g, int type, int version, int b, void *const *p, const 
     if (!group_kind(type, version, b)) return -1;
     return group_add_chunk(g, type, b, p, ctx, 0, -1);
 }
-int group_launch(TaskGroup *g, cudaStream_t s)
-{
-    return tcf2::enabled() ? tcf2::group_launch(g->g, s) : tcf::tcf_group_launch(g->g, s);
-}
+int group_launch(TaskGroup *g, cudaStream_t s) { return tcf::tcf_group_launch(g->g, s); }
 
 namespace {
 // oz_i8_f64: p[np + i] holds the slice forms of the in-operands (builtin_operand_form)

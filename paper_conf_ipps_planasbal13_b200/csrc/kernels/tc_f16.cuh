@@ -101,8 +101,7 @@ __host__ __device__ inline size_t split_bytes(int R, int K)
 }
 // byte offset of the 16-byte chunk holding elements (r, 8c .. 8c+7) of the big part; the
 // small part of the same chunk is GR * 64 bytes further (big and small of one GR-row group
-// are adjacent, so one bulk copy moves both: 32 KB for GR = 256, the CTA tile of
-// tcf_gemm_kernel; 16 KB for GR = 128, one CTA's half of the CTA-pair tile of tc_f16v2.cuh)
+// are adjacent, so one 32 KB bulk copy moves both; GR = 256, the CTA tile of tcf_gemm_kernel)
 constexpr int SPLIT_HALF = 256 * 64;
 template <int GR = 256>
 __host__ __device__ inline size_t split_chunk_off(int Rp, int r, int c)
@@ -557,7 +556,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
 
 // ---------------------------------------------------------------- host launchers
 // Split forms: X is R x K row-major (ld) -> row form; X is K x R row-major -> row form of X^T.
-// gr: row group of the layout (256: tcf_gemm_kernel, 128: the CTA-pair kernel of tc_f16v2.cuh)
+// gr: row group of the layout (256 = the CTA tile of tcf_gemm_kernel; 128 also supported)
 inline int split_rows(const float *X, int R, int K, int ld, void *out, cudaStream_t s, int gr = 256)
 {
     if (R <= 0 || K <= 0 || K % 32 || ld % 4 || (gr != 256 && gr != 128)) return -1;
