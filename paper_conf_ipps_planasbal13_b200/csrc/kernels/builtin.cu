@@ -24,6 +24,7 @@
 #include <tuple>
 #include <type_traits>
 
+#include "blk_chol.cuh"
 #include "dmma_gemm.cuh"
 #include "kernels.hpp"
 #include "simt_chol.cuh"
@@ -67,7 +68,10 @@ struct SimtEngine {
     }
     static int trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
     {
-        return blocked_trsm<Tin, Tp, SimtEngine>(rows, n, L, ldl, X, ldx, s, ctx);
+        if constexpr (std::is_same<Tin, float>::value && std::is_same<Tacc, float>::value)
+            return blk::trsm(rows, n, L, ldl, X, ldx, s, ctx);   // one launch, sub-tile DAG (blk_chol.cuh)
+        else
+            return blocked_trsm<Tin, Tp, SimtEngine>(rows, n, L, ldl, X, ldx, s, ctx);
     }
 };
 template <typename Tin>
@@ -141,6 +145,8 @@ int run_family(int type, int b, void *const *p, int *info, cudaStream_t s, const
     case VS_T_POTRF:  // A = L L^T in place        (L697-699, R9)
         if constexpr (std::is_same<E, TcEngine>::value)
             return tc::tc_potrf(b, (float *)p[0], b, 0, info, s, ctx);   // single launch (tc_panel.cuh)
+        else if constexpr (std::is_same<E, SimtEngine<float, float>>::value)
+            return blk::potrf(b, (float *)p[0], b, 0, info, s, ctx);     // single launch (blk_chol.cuh)
         else
             return potrf_rec<Tin, E>((Tin *)p[0], b, b, 0, info, s, ctx);
     }
@@ -207,12 +213,12 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
     if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
     if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
     if (form == FORM_INV_L) {
-        // X = I L^{-T} by the substitution kernel of tc_3xtf32 (tc_panel), then the row
+        // X = I L^{-T} by the sub-tile DAG substitution kernel (blk_chol.cuh), then the row
         // split form of X^T = inv(L): reading R31 (TRSM of tc_3xf16 multiplies by it)
         float *X = (float *)((uint8_t *)dst + (tcf::split_bytes(b, b) + 255) / 256 * 256);
         count_launch();
         tcf::eye_kernel<<<148, 256, 0, s>>>(X, b);
-        if (tc::tc_trsm(b, b, (const float *)src, b, X, b, s)) return -1;
+        if (blk::trsm(b, b, (const float *)src, b, X, b, s)) return -1;
         return tcf::split_cols(X, b, b, b, dst, s);
     }
     return -1;
