@@ -105,7 +105,8 @@ enum {
                              7 int8 slices under a power-of-two row scale (a cached "slice form",
                              like tc_3xf16's split form), the 28 slice products with i + j <= 8
                              accumulated exactly in int32 TMEM (one accumulator per diagonal),
-                             combined in fp64; MATMUL, GEMM_NT, SYRK; no POTRF / TRSM */
+                             combined in fp64; MATMUL, GEMM_NT, SYRK, and TRSM as X = B inv(L)^T
+                             with the slice form of inv(L) (like tc_3xf16's R31); no POTRF */
     VS_NUM_BUILTIN_VERSIONS = 7
 };
 
@@ -172,6 +173,19 @@ typedef struct {
                           host-mapped ready ring, which the host reads instead of counting
                           predecessors.  0: the host releases successors.  VS_TRACKER=device /
                           host overrides */
+    const char *trace_path; /* non-NULL: every vs_wait_* (and vs_decision_log_clear) appends the
+                          decision-log records completed since the previous append to this file
+                          as JSON lines {"task", "type", "version", "worker", "phase",
+                          "t_decide_ns", "t_start_ns", "t_end_ns"}; the string is copied */
+    /* Device memory for tile replicas and operand forms (slabs of >= 1 GiB, or the request
+     * size when that fails) comes from dev_alloc(cuda_device, bytes, alloc_user) when set
+     * (e.g. a framework's caching allocator; NULL = out of memory) and is returned with
+     * dev_free(cuda_device, ptr, alloc_user) at vs_destroy (dev_alloc without dev_free: never
+     * returned).  NULL: cudaMalloc / cudaFree.  Control structures of the runtime (execution
+     * records, rings, completion words) always use the CUDA allocator. */
+    void *(*dev_alloc)(int device, size_t bytes, void *user);
+    void (*dev_free)(int device, void *ptr, void *user);
+    void *alloc_user;
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,
@@ -218,8 +232,8 @@ int vs_version_add(vs_rt rt, vs_type_id type, const char *name, uint32_t gpu_mas
  * set in version_mask (bit = VS_V_*).  Versions each type actually gets:
  *   VS_F32: SIMT_F32, TC_3XTF32, F64IN_F32IO for all five types; TC_3XF16 for MATMUL,
  *           GEMM_NT, SYRK and TRSM (by inverse, R31) — not POTRF.
- *   VS_F64: DFMA_F64, DMMA_F64 for all five types; OZ_I8_F64 for MATMUL, GEMM_NT, SYRK —
- *           not POTRF / TRSM.
+ *   VS_F64: DFMA_F64, DMMA_F64 for all five types; OZ_I8_F64 for MATMUL, GEMM_NT, SYRK and
+ *           TRSM (by inverse) — not POTRF.
  * out_types[VS_T_*] receives the type ids.  Version INDICES are per type: inside each type
  * the kept versions are numbered 0, 1, ... in increasing VS_V_* order, skipping those the type
  * does not get, so the same index may name different versions in different types (e.g. with
@@ -370,7 +384,8 @@ int vs_tile_run(int type, int version, int b, void *const *ptrs, int *dinfo, voi
  * task.  Form 3 (TRSM of VS_V_TC_3XF16) = row split form of inv(L) for the lower triangle L
  * of the tile (reading R31).  Forms 4 / 5 / 6 (VS_V_OZ_I8_F64) = int8 slice form of the
  * rows (A role) / of the columns (matmul B) / of the rows in the B role of an NT product, of a
- * b x b fp64 tile.  VS_E_INVAL on bad arguments. */
+ * b x b fp64 tile; form 7 (TRSM of VS_V_OZ_I8_F64) = the B-role slice form of the rows of inv(L)
+ * for the lower triangle L of a b x b fp64 tile.  VS_E_INVAL on bad arguments. */
 int vs_operand_form(int type, int version, int param);
 int64_t vs_form_bytes(int form, int b);
 int vs_form_make(int form, int b, const void *src, void *dst, void *stream);

@@ -42,7 +42,13 @@ class vs_config(Structure):
                 ("mode", c_int), ("replay", c_int), ("flush", c_int), ("lookahead", c_int), ("priority", c_int),
                 ("group_ratio_permille", c_int), ("ewma_weight", c_int), ("locality_gbps", c_int),
                 ("queue_depth", c_int), ("group_tasks", c_int), ("group_wait_us", c_int), ("group_hold", c_int),
-                ("device_release", c_int)]
+                ("device_release", c_int), ("trace_path", c_char_p), ("dev_alloc", c_void_p), ("dev_free", c_void_p),
+                ("alloc_user", c_void_p)]
+
+
+# device allocator hooks of vs_config (dev_alloc / dev_free)
+VS_DEV_ALLOC_FN = ctypes.CFUNCTYPE(c_void_p, c_int, c_size_t, c_void_p)
+VS_DEV_FREE_FN = ctypes.CFUNCTYPE(None, c_int, c_void_p, c_void_p)
 
 
 class vs_stats_t(Structure):
@@ -157,9 +163,18 @@ def _ids(seq, ctype=c_int64):
 
 # ------------------------------------------------------------------ thin wrappers
 def vs_config_default(**kw) -> vs_config:
+    """vs_config with defaults, keyword overrides on top.  trace_path: str; dev_alloc /
+    dev_free: ctypes callbacks (VS_DEV_ALLOC_FN / VS_DEV_FREE_FN) kept alive by the config."""
     c = vs_config()
     lib().vs_config_default(ctypes.byref(c))
+    c._keep = []
     for k, v in kw.items():
+        if k == "trace_path" and isinstance(v, str):
+            v = v.encode()
+            c._keep.append(v)
+        elif k in ("dev_alloc", "dev_free") and v is not None and not isinstance(v, int):
+            c._keep.append(v)
+            v = ctypes.cast(v, c_void_p).value
         setattr(c, "lambda_" if k == "lam" else k, v)
     return c
 
@@ -244,7 +259,7 @@ class Runtime:
 
     def __init__(self, cfg: vs_config | None = None, **kw):
         L = lib()
-        self.cfg = cfg if cfg is not None else vs_config_default(**kw)
+        self.cfg = cfg if cfg is not None else vs_config_default(**kw)   # keeps the callbacks alive
         h = c_void_p()
         r = L.vs_create(ctypes.byref(self.cfg), ctypes.byref(h))
         if r:

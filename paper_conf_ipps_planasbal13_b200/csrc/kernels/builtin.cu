@@ -40,6 +40,12 @@ namespace vsk {
 
 namespace {
 
+__global__ void eye64_kernel(double *X, int n)
+{
+    for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < (int64_t)n * n; i += (int64_t)gridDim.x * blockDim.x)
+        X[i] = (i / n == i % n) ? 1.0 : 0.0;
+}
+
 template <typename Tin, typename Tp, class Gemm>
 int blocked_trsm(int rows, int n, const Tin *L, int ldl, Tin *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
 {
@@ -165,7 +171,7 @@ bool builtin_supported(int type, int version, int b)
     if (type < 0 || type >= VS_NUM_BUILTIN_TYPES) return false;
     if (version < 0 || version >= VS_NUM_BUILTIN_VERSIONS) return false;
     if (version == VS_V_TC_3XF16 && type == VS_T_POTRF) return false;
-    if (version == VS_V_OZ_I8_F64 && (type == VS_T_POTRF || type == VS_T_TRSM)) return false;
+    if (version == VS_V_OZ_I8_F64 && type == VS_T_POTRF) return false;
     if (b && (b % 64 != 0 || b < 64 || b > 4096)) return false;
     return true;
 }
@@ -183,6 +189,7 @@ int builtin_operand_form(int type, int version, int param)
         case VS_T_MATMUL: return param == 0 ? FORM_OZ_ROWS : param == 1 ? FORM_OZ_COLS : FORM_RAW;
         case VS_T_GEMM_NT: return param == 0 ? FORM_OZ_ROWS : param == 1 ? FORM_OZ_ROWS_B : FORM_RAW;
         case VS_T_SYRK: return param == 0 ? FORM_OZ_ROWS : FORM_RAW;
+        case VS_T_TRSM: return param == 0 ? FORM_OZ_INV_L : FORM_OZ_ROWS;   // X = B inv(L)^T
         }
         return FORM_RAW;
     }
@@ -201,6 +208,7 @@ size_t form_bytes(int form, int b)
     if (form == FORM_RAW) return 0;
     if (form == FORM_OZ_ROWS || form == FORM_OZ_COLS || form == FORM_OZ_ROWS_B)
         return (oz::form_bytes(b, b) + 255) / 256 * 256;
+    if (form == FORM_OZ_INV_L) return (oz::form_bytes(b, b) + 255) / 256 * 256 + (size_t)b * b * 8;   // + fp64 scratch
     const size_t sb = (tcf::split_bytes(b, b) + 255) / 256 * 256;
     return form == FORM_INV_L ? sb + (size_t)b * b * 4 : sb;   // + fp32 scratch for inv(L)^T
 }
@@ -210,6 +218,15 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
     if (form == FORM_OZ_ROWS) return oz::make_slices((const double *)src, b, b, b, 1, 128, dst, s);
     if (form == FORM_OZ_ROWS_B) return oz::make_slices((const double *)src, b, b, b, 1, 64, dst, s);
     if (form == FORM_OZ_COLS) return oz::make_slices((const double *)src, b, b, 1, b, 64, dst, s);
+    if (form == FORM_OZ_INV_L) {
+        // X = I L^{-T} (fp64, the blocked DMMA substitution of dmma_f64), then the slice form of
+        // the columns of X = the rows of inv(L) in the B role
+        double *X = (double *)((uint8_t *)dst + (oz::form_bytes(b, b) + 255) / 256 * 256);
+        count_launch();
+        eye64_kernel<<<148, 256, 0, s>>>(X, b);
+        if (DmmaEngine<double>::trsm(b, b, (const double *)src, b, X, b, s, TaskCtx())) return -1;
+        return oz::make_slices(X, b, b, 1, b, 64, dst, s);
+    }
     if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
     if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
     if (form == FORM_INV_L) {
@@ -262,9 +279,10 @@ namespace {
 int run_oz(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
 {
     switch (type) {
-    case VS_T_MATMUL: return oz::oz_gemm<false, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, ctx);   // C += A B
-    case VS_T_GEMM_NT: return oz::oz_gemm<true, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, ctx);  // C -= A B^T
-    case VS_T_SYRK: return oz::oz_gemm<true, true, 128>(b, b, b, p[2], p[2], (double *)p[1], b, s, ctx);     // C -= A A^T
+    case VS_T_MATMUL: return oz::oz_gemm<false, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, false, ctx);   // C += A B
+    case VS_T_GEMM_NT: return oz::oz_gemm<true, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, false, ctx);  // C -= A B^T
+    case VS_T_SYRK: return oz::oz_gemm<true, true, 128>(b, b, b, p[2], p[2], (double *)p[1], b, s, false, ctx);   // C -= A A^T
+    case VS_T_TRSM: return oz::oz_gemm<false, false, 64>(b, b, b, p[3], p[2], (double *)p[1], b, s, true, ctx);  // X = B inv(L)^T
     }
     return -1;
 }

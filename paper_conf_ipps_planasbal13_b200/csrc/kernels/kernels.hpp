@@ -74,8 +74,11 @@ int builtin_elem_bytes(int version);
 // FORM_OZ_ROWS / FORM_OZ_COLS / FORM_OZ_ROWS_B: int8 slice forms of the rows (A role,
 // 128-row groups) / columns (matmul B, 64-row groups) / rows (NT B role, 64-row groups) of
 // an fp64 tile (oz_i8_f64, tc_oz.cuh).
+// FORM_OZ_INV_L: int8 slice form (B role) of the rows of inv(L) for the lower triangle L of an
+// fp64 tile (TRSM of oz_i8_f64 as X = B inv(L)^T, like tc_3xf16's FORM_INV_L).
 enum { FORM_RAW = 0, FORM_SPLIT_ROWS = 1, FORM_SPLIT_COLS = 2, FORM_INV_L = 3, FORM_OZ_ROWS = 4, FORM_OZ_COLS = 5,
-       FORM_OZ_ROWS_B = 6, NUM_FORMS = 7 };
+       FORM_OZ_ROWS_B = 6, FORM_OZ_INV_L = 7, NUM_FORMS = 8 };
+inline bool form_is_f64(int f) { return f == FORM_OZ_ROWS || f == FORM_OZ_COLS || f == FORM_OZ_ROWS_B || f == FORM_OZ_INV_L; }
 int builtin_nparams(int type);
 int builtin_operand_form(int type, int version, int param);
 size_t form_bytes(int form, int b);

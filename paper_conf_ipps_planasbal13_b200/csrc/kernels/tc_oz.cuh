@@ -192,7 +192,7 @@ __device__ __forceinline__ void bulk_g2s(uint32_t dst, const void *src, uint32_t
 template <bool NEG, bool LOWER, int GB>
 __global__ void __launch_bounds__(NTHREADS, 1)
     oz_gemm_kernel(int M, int N, int K, const uint8_t *__restrict__ Af, const uint8_t *__restrict__ Bf,
-                   double *__restrict__ C, int ldc, TaskCtx ctx)
+                   double *__restrict__ C, int ldc, int beta0, TaskCtx ctx)
 {
     extern __shared__ uint8_t smem_raw[];
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
@@ -282,7 +282,7 @@ __global__ void __launch_bounds__(NTHREADS, 1)
                 const int grow = m0 + 32 * q + r;
                 if (grow < M && gcol < N && (!LOWER || gcol <= grow)) {
                     double *cp = C + (int64_t)grow * ldc + gcol;
-                    *cp = *cp + stg[r * EPI_LD + lane] * sbl;
+                    *cp = (beta0 ? 0.0 : *cp) + stg[r * EPI_LD + lane] * sbl;
                 }
             }
             __syncwarp();
@@ -348,8 +348,9 @@ inline int make_slices(const double *X, int R, int K, int64_t sr, int64_t sk, in
 
 // C (M x N, ldc) += s * A * B'^T with A (G = 128) and B' (G = GB) in slice form (K a
 // multiple of 64).
+// beta0: C = s A B^T (C_in not read; the TRSM by inverse overwrites its right-hand side)
 template <bool NEG, bool LOWER, int GB>
-inline int oz_gemm(int M, int N, int K, const void *Af, const void *Bf, double *C, int ldc, cudaStream_t s,
+inline int oz_gemm(int M, int N, int K, const void *Af, const void *Bf, double *C, int ldc, cudaStream_t s, bool beta0,
                    const TaskCtx &ctx = TaskCtx())
 {
     if (M <= 0 || N <= 0) return 0;
@@ -365,7 +366,7 @@ inline int oz_gemm(int M, int N, int K, const void *Af, const void *Bf, double *
     TaskCtx c = ctx_for(ctx, oz_gemm_kernel<NEG, LOWER, GB>, NTHREADS, SMEM);
     c.ncta = grid.x * grid.y;
     count_launch();
-    oz_gemm_kernel<NEG, LOWER, GB><<<grid, NTHREADS, SMEM, s>>>(M, N, K, (const uint8_t *)Af, (const uint8_t *)Bf, C, ldc, c);
+    oz_gemm_kernel<NEG, LOWER, GB><<<grid, NTHREADS, SMEM, s>>>(M, N, K, (const uint8_t *)Af, (const uint8_t *)Bf, C, ldc, beta0 ? 1 : 0, c);
     return 0;
 }
 

@@ -42,6 +42,21 @@
 namespace vsk {
 namespace tc {
 
+// Optional per-CTA, per-panel timeline (a probe builds with -DVS_PANEL_TRACE):
+// [cta][panel][0] epilogue: flag seen, [1] L_JJ staged, [2] accumulator ready, [3] panel solved,
+// [4] producer: flag seen (potrf), [5] producer: last k-block issued
+#ifdef VS_PANEL_TRACE
+__device__ unsigned long long g_panel_trace[32][32][6];
+#define PANEL_T(J, i)                                                                  \
+    do {                                                                               \
+        unsigned long long t_;                                                         \
+        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_));                         \
+        g_panel_trace[blockIdx.x & 31][(J) & 31][i] = t_;                              \
+    } while (0)
+#else
+#define PANEL_T(J, i)
+#endif
+
 constexpr int PNL = 128;   // panel width (= BM: panel J's diagonal block is CTA J's rows)
 constexpr int PSB = 16;    // solve sub-block
 constexpr int kFlagSlots = 4096;
@@ -220,6 +235,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 if (t == 0) wait_flag(&flags[J], tag | (unsigned long long)J);
                 asm volatile("bar.sync 1, 128;" ::: "memory");
             }
+            if (t == 0) PANEL_T(J, 4);
             // first k-block holding panel J-1's columns (overlap = 0: the whole panel waits)
             const int kb_new = overlap ? nk - P / BK : 0;
             constexpr uint32_t idesc = make_idesc(BM, P, false, false);
@@ -302,6 +318,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     if (kb + 3 < nk) load(ra1, rb1, kb + 3);
                 }
             }
+            if (t == 0) PANEL_T(J, 5);
         }
     } else {
         // =================================================== epilogue (warps 4-7)
@@ -320,6 +337,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     if (e == 0) wait_flag(&flags[J], tag | (unsigned long long)(J + 1));
                     bar_epi();
                 }
+                if (e == 0) PANEL_T(J, 0);
                 // stage L_JJ^T: rows q of L_JJ, coalesced in c = e; batched loads
 #pragma unroll 1
                 for (int q0 = 0; q0 < ncols; q0 += 32) {
@@ -334,6 +352,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 }
                 if (e < ncols) Lr[e] = rcp_approx(Lt[e * LD + e]);   // this thread's own store
                 bar_epi();
+                if (e == 0) PANEL_T(J, 1);
             }
             // b values of sub-block 0 (the tile's current values of the panel columns)
             float4 bq[4], bn[4];
@@ -343,6 +362,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 mbar_wait(&accf[J & 1], (accn >> (J & 1)) & 1u);
                 accn ^= 1u << (J & 1);
                 tc_fence_after();
+                if (e == 0) PANEL_T(J, 2);
             } else {
                 float z[16];
 #pragma unroll
@@ -448,6 +468,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
 #pragma unroll
                 for (int q = 0; q < 4; q++) bq[q] = bn[q];
             }
+            if (e == 0) PANEL_T(J, 3);
             // panel J of these rows: visible at L2 (own producers, other CTAs), TMEM reads done
             __threadfence();
             tc_fence_before();

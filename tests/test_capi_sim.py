@@ -390,3 +390,31 @@ def test_version_mask_must_name_a_configured_gpu():
         rt.vs_submit(t, [rt.vs_data_register(_fake_ptr(0, 4096), 0, 4096)])   # no version at all
     rt.vs_version_add(t, "gpu1", 1 << 1)
     assert rt.vs_submit(t, [rt.vs_data_register(_fake_ptr(0, 4096), 0, 4096)]) == 0
+
+
+def test_trace_path_jsonl_matches_decision_log(tmp_path):
+    """vs_config.trace_path (§8(b)): each wait appends the decisions completed since the last one
+    as JSON lines, identical to vs_decision_log."""
+    import json
+    path = str(tmp_path / "trace.jsonl")
+    rt = _sim(slots=2, lam=1, trace_path=path)
+    t = rt.vs_type_create("MATMUL", [vs.VS_IN, vs.VS_IN, vs.VS_INOUT])
+    for v in range(2):
+        rt.vs_version_add(t, "v%d" % v, ALL)
+    nb = 4096
+    ids = [rt.vs_data_register(_fake_ptr(i, nb), 0, nb) for i in range(12)]
+    rt.vs_app_matmul(t, 2, 2, 2, ids[:4], ids[4:8], ids[8:])
+    rt.vs_replay_set(t, 3 * nb, 0, 3000)
+    rt.vs_replay_set(t, 3 * nb, 1, 1000)
+    rt.vs_wait_all()
+    rt.vs_app_matmul(t, 2, 2, 2, ids[:4], ids[4:8], ids[8:])
+    rt.vs_wait_all_noflush()
+    lines = [json.loads(x) for x in open(path)]
+    log = rt.vs_decision_log()
+    assert len(lines) == len(log) == 16
+    for rec, r in zip(lines, log):
+        assert (rec["task"], rec["worker"], rec["phase"], rec["t_decide_ns"], rec["t_start_ns"], rec["t_end_ns"]) == \
+            (r[0], r[2], r[6], r[3], r[4], r[5])
+        assert rec["type"] == "MATMUL" and rec["version"] == "v%d" % r[1]
+    rt.vs_decision_log_clear()
+    assert len(open(path).read().splitlines()) == 16    # nothing written twice

@@ -360,3 +360,38 @@ def test_device_release_matmul_and_cholesky(gpu):
     assert rt.vs_stats().device_released == st.device_released + 48
     assert oracle.relF(vsgen.from_tiles(T[2].cpu().numpy()), oracle.matmul(A, B)) <= 1e-5
     rt.close()
+
+
+def test_dev_alloc_hooks_use_the_callers_allocator(gpu):
+    """vs_config.dev_alloc / dev_free (§8(b)): replicas and operand forms come from the caller's
+    allocator — here torch's caching allocator — and are returned at vs_destroy."""
+    torch = _torch()
+    calls = {"alloc": 0, "free": 0, "bytes": 0}
+    live = {}
+
+    def alloc(dev, nbytes, user):
+        calls["alloc"] += 1
+        calls["bytes"] += nbytes
+        p = torch.cuda.caching_allocator_alloc(nbytes, device=dev)
+        live[p] = nbytes
+        return p
+
+    def free(dev, ptr, user):
+        calls["free"] += 1
+        torch.cuda.caching_allocator_delete(ptr)
+        live.pop(ptr)
+
+    fa, ff = vs.VS_DEV_ALLOC_FN(alloc), vs.VS_DEV_FREE_FN(free)
+    rt = vs.Runtime(vs.vs_config_default(lam=1, slots_per_gpu=2, dev_alloc=fa, dev_free=ff))
+    N, b = 512, 128
+    nt = N // b
+    types = rt.vs_register_builtins(vs.VS_F32, (1 << vs.VS_V_TC_3XTF32) | (1 << vs.VS_V_TC_3XF16))
+    A, B = vsgen.uniform(3, N, N), vsgen.uniform(1003, N, N)
+    T = [torch.from_numpy(vsgen.to_tiles(x, b)).pin_memory() for x in (A, B, np.zeros((N, N), np.float32))]
+    ids = [[rt.vs_data_register(X[i, j].data_ptr(), -1, b * b * 4) for i in range(nt) for j in range(nt)] for X in T]
+    rt.vs_app_matmul(types[vs.VS_T_MATMUL], nt, nt, nt, *ids)
+    rt.vs_wait_all()
+    assert calls["alloc"] >= 1 and calls["bytes"] >= 48 * b * b * 4      # host-homed tiles got device replicas
+    assert oracle.relF(vsgen.from_tiles(T[2].numpy()), oracle.matmul(A, B)) <= 1e-5
+    rt.close()
+    assert calls["free"] == calls["alloc"] and not live

@@ -181,7 +181,7 @@ def test_oz_i8_f64_row_scales_and_componentwise_bound(gpu, ttype):
 
 
 # ------------------------------------------------------------------ trsm / potrf
-@pytest.mark.parametrize("version", F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS)
+@pytest.mark.parametrize("version", F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS + [vs.VS_V_OZ_I8_F64])
 @pytest.mark.parametrize("b", [64, 128, 192, 512, 1024])
 def test_trsm_tile(gpu, version, b):
     dt = _dt(version)
