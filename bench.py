@@ -61,14 +61,15 @@ def bench_config(vs, **over):
     return vs.vs_config_default(**kw)
 
 
-def ncu_traffic(path=os.path.join(ROOT, "profiles", "r01s3_ncu_full_tcf.csv")):
+def ncu_traffic(path=os.path.join(ROOT, "profiles", "r02_ncu_full_tcf_bench.csv")):
     """dram__bytes_read.sum + dram__bytes_write.sum of the committed ncu --set full capture of
-    one tcf_gemm_kernel launch inside the bench (bytes per launch), or None."""
+    one steady-state tcf_gemm_kernel<24,1> launch inside the bench (8 tasks, 128 CTAs; bytes per
+    launch), or None."""
     import csv
     scale = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}
     try:
         tot = 0.0
-        for m, unit, v in list(csv.reader(open(path)))[1:]:
+        for m, unit, v in [r for r in csv.reader(open(path)) if len(r) == 3][1:]:
             if m in ("dram__bytes_read.sum", "dram__bytes_write.sum"):
                 tot += float(v) * scale.get(unit, 1)
         return int(tot)
@@ -278,7 +279,7 @@ def task_flops(type_name, b):
             "POTRF": b ** 3 / 3.0}[t]
 
 
-def roofline(log, groups, ms, world):
+def roofline(log, groups, ms, world, launch_of=None):
     pk, pk_kind = peaks()
     tf32_peak = pk.get("bf16_tflops_sustained", pk["bf16_tflops"]) * 0.5   # TF32 = 1/2 BF16 (nominal ratio)
     tnames = {g["type"]: g["type_name"] for g in groups}
@@ -305,6 +306,27 @@ def roofline(log, groups, ms, world):
     dom = max(per, key=lambda k: per[k]["flops"])
     d = per[dom]
     union = union_ns(d["iv"])
+    # per launch (the contract's definition): each launch's hardware flops / its own duration
+    # (first task start -> last task end of the tasks it ran), averaged over the launches
+    per_launch = None
+    if launch_of is not None:
+        ln = {}
+        for rec, lno in zip(log, launch_of):
+            (task, v, w, td, ts, te, ph, ty) = rec
+            tname, vname = tnames[ty], vnames[ty][v]
+            kname = "tcf_gemm_kernel" if vname == "tc_3xf16" and not tname.startswith("POTRF") else "%s/%s" % (tname, vname)
+            if kname != dom or lno < 0:
+                continue
+            e = ln.setdefault(lno, [0.0, ts, te, 0])
+            e[0] += task_flops(tname, tile_b[ty])
+            e[1], e[2], e[3] = min(e[1], ts), max(e[2], te), e[3] + 1
+        if ln:
+            hw_l = 3.0 if d["version"] in ("tc_3xtf32", "tc_3xf16") else 1.0
+            fl = sum(x[0] for x in ln.values()) * hw_l
+            dur = sum(x[2] - x[1] for x in ln.values())
+            per_launch = {"launches": len(ln), "tasks_per_launch": round(sum(x[3] for x in ln.values()) / len(ln), 2),
+                          "avg_launch_us": round(dur / len(ln) / 1e3, 2),
+                          "achieved": round(fl / (dur * 1e-9) / 1e12, 2)}
     f16_peak = pk.get("bf16_tflops_sustained", pk["bf16_tflops"])            # fp16 dense = bf16 dense rate
     tc_peak = {"tc_3xtf32": (tf32_peak, "%s bf16_tflops_sustained x 0.5 (TF32/BF16 nominal ratio)" % pk_kind),
                "tc_3xf16": (f16_peak, "%s bf16_tflops_sustained (fp16 = bf16 dense rate)" % pk_kind)}
@@ -318,15 +340,21 @@ def roofline(log, groups, ms, world):
     # task / (step time x that version's peak), summed over versions
     frac_step = sum(3.0 * v["flops"] / tc_peak[k[1]][0] for k, v in per_tv.items() if k[1] in tc_peak) / (ms * 1e-3) / 1e12
     traffic = ncu_traffic() if dom == "tcf_gemm_kernel" else None
+    if per_launch:
+        per_launch["frac"] = round(per_launch["achieved"] / peak, 4)
     roof = {"bound": bound, "kernel": dom, "tasks": d["n"], "achieved": round(achieved, 2), "peak": round(peak, 1),
             "unit": "TFLOP/s", "frac": round(achieved / peak, 4), "traffic": traffic,
-            "traffic_note": ("DRAM bytes of one captured launch (ncu --set full, profiles/r01s3_ncu_full_tcf.csv: "
-                             "one SYRK b=1024 task; algorithmic 4 MiB form + 2.5 MiB C read + 2.5 MiB C written, "
-                             "C write-back happens after the kernel)") if traffic else None,
+            "traffic_note": ("DRAM bytes of one captured steady-state launch (ncu --set full, "
+                             "profiles/r02_ncu_full_tcf_bench.csv: tcf_gemm_kernel<24,1>, 8 MATMUL/GEMM_NT tasks, "
+                             "128 CTAs; algorithmic reads 8 x (A form 4 MiB + B form 4 MiB + C 4 MiB) = 100.7 MB, "
+                             "writes 33.6 MB, most of which leave L2 after the kernel)") if traffic else None,
+            "per_launch": per_launch,
             "peak_source": src,
             "how": "hardware MMA flops (3x the algorithmic flops of its tasks: 2b^3 matmul/gemm, b^3 syrk/trsm) of "
                    "every task this kernel ran in the timed steps / union of their device-recorded execution "
-                   "intervals (%globaltimer, task_ctx.cuh)"}
+                   "intervals (%globaltimer, task_ctx.cuh); per_launch: the same flops / the sum of each launch's "
+                   "own duration (first task start to last task end), i.e. the average launch rate, which "
+                   "counts the time concurrent launches on other streams share the SMs against each launch"}
     counts = {"%s/%s" % k[:2]: v["n"] for k, v in sorted(per_tv.items())}
     return roof, frac_step, counts
 
@@ -590,10 +618,11 @@ def main():
         ms = max(gather(ms))
     st1 = rt.vs_stats()
     log = rt.vs_decision_log()
+    launch_of = rt.vs_decision_launches()
     groups = rt.vs_group_stats()
     ms_step = ms / args.steps
     gflops = wl.flops * args.steps / (ms * 1e-3) / 1e9       # one problem, sharded over the ranks
-    roof, frac_step, version_counts = roofline(log, groups, ms, 1)
+    roof, frac_step, version_counts = roofline(log, groups, ms, 1, launch_of)
     launches = st1.kernel_launches - st0.kernel_launches
     if dist is not None:
         launches = sum(gather(int(launches)))

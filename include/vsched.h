@@ -330,6 +330,9 @@ typedef struct {
     int64_t t_decide_ns;       /* virtual (run-ahead / sim) or host clock (ready) */
     int64_t t_start_ns, t_end_ns; /* sim: virtual clock; gpu: GPU timeline of the version's
                                      start/end events (ns since runtime creation) */
+    int64_t launch;               /* gpu: number of the kernel launch that ran a built-in
+                                     version's task (tasks of one grouped launch share it;
+                                     multi-kernel versions: the first), -1 otherwise */
 } vs_decision_t;
 /* Host wall-clock time at which each decision-log entry's task was enqueued on its
  * stream, on the t_start_ns timeline (system clock minus the same origin: the GPU's

@@ -68,7 +68,7 @@ class vs_group_stat_t(Structure):
 
 class vs_decision_t(Structure):
     _fields_ = [("task", c_int64), ("version", c_int32), ("worker", c_int32), ("phase", c_int32), ("type", c_int32),
-                ("t_decide_ns", c_int64), ("t_start_ns", c_int64), ("t_end_ns", c_int64)]
+                ("t_decide_ns", c_int64), ("t_start_ns", c_int64), ("t_end_ns", c_int64), ("launch", c_int64)]
 
 
 VS_LAUNCH_FN = ctypes.CFUNCTYPE(c_int, POINTER(c_void_p), POINTER(c_int64), c_int, c_void_p, c_size_t, c_void_p,
@@ -365,6 +365,14 @@ class Runtime:
         lib().vs_decision_log(self.h, buf, n.value, ctypes.byref(n))
         return [(r.task, r.version, r.worker, r.t_decide_ns, r.t_start_ns, r.t_end_ns, r.phase, r.type)
                 for r in buf[:n.value]]
+
+    def vs_decision_launches(self):
+        """vs_decision_t.launch of every record (kernel launch number; grouped tasks share one)."""
+        n = c_int64()
+        lib().vs_decision_log(self.h, None, 0, ctypes.byref(n))
+        buf = (vs_decision_t * max(1, n.value))()
+        lib().vs_decision_log(self.h, buf, n.value, ctypes.byref(n))
+        return [r.launch for r in buf[:n.value]]
 
     def vs_decision_issue_ns(self):
         n = c_int64()
