@@ -19,9 +19,10 @@
 //        x = b - acc[sb]  (b = the tile's current values, prefetched one sub-block ahead);
 //        TRSM / POTRF below the diagonal: forward substitution against L_JJ staged
 //          (transposed) in shared memory (x_c = t_c / l_cc; t_j -= x_c l_jc);
-//        POTRF diagonal CTA (CTA J holds panel J's diagonal block): right-looking
-//          factorisation column by column, the pivot row publishes l_cc = sqrt(t_c),
-//          every lower row scales and publishes l_ic (two named barriers per column);
+//        POTRF diagonal CTA (CTA J holds panel J's diagonal block): per 16-column
+//          sub-block, the warp holding its 16 diagonal rows factors them with shuffles
+//          (l_cc = sqrt(t_c), x = t / l, t_j -= x l_jc), publishes L_sb, and the rows below
+//          solve against it (two named barriers per sub-block; round 1: two per column);
 //        store x; acc[t] += x L[t, sb]^T for the later sub-blocks t (tcgen05.ld/st).
 // Roles: warps 0-3 producers (LDG -> split big/small -> 128B-swizzled K-major smem); warp 0
 // also allocates TMEM and, once all four producer warps filled a stage, issues its MMAs;
@@ -186,8 +187,6 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     float *Lt = reinterpret_cast<float *>(smem + STAGES * G::STAGE);   // Lt[c * LD + j] = L_JJ[j][c]
     __shared__ float Lr[P];       // reciprocals of the diagonal of L_JJ
-    __shared__ float colbuf[BM];  // POTRF diagonal CTA: published column
-    __shared__ float pivot;
     uint64_t *full = (uint64_t *)((uint8_t *)Lt + G::LT_BYTES);
     uint64_t *empty = full + STAGES;
     uint64_t *accf = empty + STAGES;   // [2]: accumulator of panel parity b complete
@@ -387,30 +386,57 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     x[4 * q + 3] = bq[q].w - x[4 * q + 3];
                 }
                 if (factor) {
-#pragma unroll
-                    for (int c = 0; c < PSB; c++) {
-                        const int pr = sb * PSB + c;   // pivot row / column within the block
-                        if (e == pr) {
-                            const float piv = x[c];
-                            if (!(piv > 0.f) && info) atomicCAS(info, 0, k_base + c0 + pr + 1);
-                            x[c] = sqrtf(piv);
-                            pivot = x[c];
+                    // the 16 x 16 diagonal sub-block is factored by the warp holding its rows,
+                    // with shuffles (no block barrier per column); its L is published in Lt/Lr,
+                    // then every row below solves against it exactly as the other CTAs' rows do
+                    // (same operations and operands as a column-by-column right-looking sweep:
+                    // l = sqrt(pivot), x_c = t_c / l by rcp + Newton, t_j -= x_c l_jc)
+                    const int d0 = sb * PSB, lb = d0 & 31, r = e - d0;
+                    const bool drow = r >= 0 && r < PSB;
+                    if ((e >> 5) == (d0 >> 5)) {
+                        float dg = 1.f;   // this row's diagonal l_rr (no dynamic index into x[])
+#pragma unroll 16
+                        for (int c = 0; c < PSB; c++) {
+                            const float piv = __shfl_sync(0xffffffffu, x[c], lb + c);
+                            const float l = sqrtf(piv);
+                            // selects, not branches: under `r == c` the compiler would rewrite
+                            // x[c] as x[r], a dynamic index that sends x[] to local memory
+                            const bool piv_row = drow && r == c;
+                            if (piv_row && !(piv > 0.f) && info) atomicCAS(info, 0, k_base + c0 + d0 + c + 1);
+                            const float xd = div_nr(x[c], l, rcp_approx(l));
+                            x[c] = piv_row ? l : ((drow && r > c) ? xd : x[c]);
+                            dg = piv_row ? l : dg;
+                            // rows below the pivot update every later column of the sub-block
+                            // (entries right of their own diagonal are never stored)
+                            const bool below = drow && r > c;
+#pragma unroll 16
+                            for (int j = 0; j < PSB; j++) {
+                                if (j > c) {
+                                    const float ljc = __shfl_sync(0xffffffffu, x[c], lb + j);
+                                    const float upd = fmaf(-x[c], ljc, x[j]);
+                                    x[j] = below ? upd : x[j];
+                                }
+                            }
                         }
-                        bar_epi();
-                        const float l = pivot;
-                        if (e > pr) {
-                            x[c] = div_nr(x[c], l, rcp_approx(l));
-                            colbuf[e] = x[c];
-                        }
-                        bar_epi();
-                        if (e > pr) {
+                        if (drow) {
 #pragma unroll
-                            for (int j = c + 1; j < PSB; j++) x[j] = fmaf(-x[c], colbuf[sb * PSB + j], x[j]);
+                            for (int c = 0; c < PSB; c++) Lt[(d0 + c) * LD + e] = x[c];
+                            Lr[e] = rcp_approx(dg);
                         }
                     }
-                    // publish this row's L_JJ values (transposed) for the cross updates
+                    bar_epi();
+                    if (r >= PSB) {
 #pragma unroll
-                    for (int c = 0; c < PSB; c++) Lt[(sb * PSB + c) * LD + e] = x[c];
+                        for (int c = 0; c < PSB; c++) {
+                            const int cc = d0 + c;
+                            x[c] = div_nr(x[c], Lt[cc * LD + cc], Lr[cc]);
+#pragma unroll
+                            for (int j = c + 1; j < PSB; j++) x[j] = fmaf(-x[c], Lt[cc * LD + d0 + j], x[j]);
+                        }
+                        // publish this row's L_JJ values (transposed) for the cross updates
+#pragma unroll
+                        for (int c = 0; c < PSB; c++) Lt[(d0 + c) * LD + e] = x[c];
+                    }
                     bar_epi();
                 } else {
 #pragma unroll
