@@ -45,9 +45,10 @@ namespace tc {
 
 // Optional per-CTA, per-panel timeline (a probe builds with -DVS_PANEL_TRACE):
 // [cta][panel][0] epilogue: flag seen, [1] L_JJ staged, [2] accumulator ready, [3] panel solved,
-// [4] producer: flag seen (potrf), [5] producer: last k-block issued
+// [4] producer: flag seen (potrf), [5] producer: last k-block issued, [6 + 2 sb] sub-block sb
+// solved (before the cross update), [7 + 2 sb] its cross update done
 #ifdef VS_PANEL_TRACE
-__device__ unsigned long long g_panel_trace[32][32][6];
+__device__ unsigned long long g_panel_trace[32][32][24];
 #define PANEL_T(J, i)                                                                  \
     do {                                                                               \
         unsigned long long t_;                                                         \
@@ -73,7 +74,10 @@ struct PanelCfg {
     static constexpr int STAGE = 2 * A_BYTES + 2 * B_BYTES; // 64 KB
     static constexpr int LD = PNL + 4;                      // Lt row stride (16-byte rows)
     static constexpr int LT_BYTES = PNL * LD * 4;           // 66 KB
-    static constexpr int SMEM = STAGES * STAGE + LT_BYTES + 1024 + 256;
+    static constexpr int XS_A = BM * 64;                    // 8 KB: 128 rows x 16 fp32 (SW64), one part
+    static constexpr int XS_B = (PNL - 16) * 64;            // 7 KB: at most 112 rows of L_JJ, one part
+    static constexpr int XS_BYTES = 2 * XS_A + 2 * XS_B;    // cross-sub-block update operands
+    static constexpr int SMEM = STAGES * STAGE + LT_BYTES + XS_BYTES + 1024 + 256;
     static constexpr int APER = BM * BK / 4 / NP;           // 8
     static constexpr int BPER = PNL * BK / 4 / NP;          // 8
 };
@@ -173,6 +177,18 @@ __device__ __forceinline__ void tmem_st16_issue(uint32_t taddr, const float (&v)
 }
 __device__ __forceinline__ void tmem_wait_st() { asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory"); }
 __device__ __forceinline__ void bar_epi() { asm volatile("bar.sync 2, 128;" ::: "memory"); }
+// UMMA shared-memory descriptor, K-major SWIZZLE_64B (layout 4): 64-byte rows, 8-row atoms of
+// 512 B (SBO), version 1 — the cross-sub-block update operands (16 fp32 of K per row)
+__device__ __forceinline__ uint64_t desc_sw64(uint32_t saddr)
+{
+    uint64_t d = 0;
+    d |= (uint64_t)((saddr & 0x3FFFF) >> 4);
+    d |= (uint64_t)(16 >> 4) << 16;
+    d |= (uint64_t)(512 >> 4) << 32;
+    d |= (uint64_t)1 << 46;
+    d |= (uint64_t)4 << 61;
+    return d;
+}
 
 template <bool POTRF>
 __global__ void __launch_bounds__(PTHREADS, 1)
@@ -187,14 +203,25 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
     float *Lt = reinterpret_cast<float *>(smem + STAGES * G::STAGE);   // Lt[c * LD + j] = L_JJ[j][c]
     __shared__ float Lr[P];       // reciprocals of the diagonal of L_JJ
-    uint64_t *full = (uint64_t *)((uint8_t *)Lt + G::LT_BYTES);
+    // XS: operands of the cross-sub-block update MMAs (1024-aligned: STAGE and LT_BYTES keep it)
+    uint8_t *xs_ab = (uint8_t *)Lt + G::LT_BYTES, *xs_as = xs_ab + G::XS_A;
+    uint8_t *xs_bb = xs_as + G::XS_A, *xs_bs = xs_bb + G::XS_B;
+    uint64_t *full = (uint64_t *)(xs_bs + G::XS_B);
     uint64_t *empty = full + STAGES;
     uint64_t *accf = empty + STAGES;   // [2]: accumulator of panel parity b complete
     uint64_t *xdone = accf + 2;        // one phase per panel: its columns solved and stored
-    uint32_t *tmem_slot = (uint32_t *)(xdone + 1);
+    uint64_t *xacc = xdone + 1;        // cross-sub-block update MMAs complete (one phase per use)
+    uint32_t *tmem_slot = (uint32_t *)(xacc + 1);
 
     const int m0 = blockIdx.x * BM;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+#ifdef VS_PANEL_TRACE
+    if (threadIdx.x == 0) {
+        unsigned smid;
+        asm volatile("mov.u32 %0, %%smid;" : "=r"(smid));
+        g_panel_trace[blockIdx.x & 31][31][23] = smid;
+    }
+#endif
     unsigned long long *flags = POTRF ? g_panel_flags[launch_id % kFlagSlots] : nullptr;
     const unsigned long long tag = launch_id << 8;
     if (threadIdx.x == 0) {
@@ -205,6 +232,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
         mbar_init(&accf[0], 1);
         mbar_init(&accf[1], 1);
         mbar_init(xdone, 4);
+        mbar_init(xacc, 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     }
     if (warp == 0) {
@@ -326,6 +354,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
         const bool rowok = row < rows;
         float *xrow = X + (int64_t)(rowok ? row : 0) * ldx;
         uint32_t accn = 0;   // bit b: parity of the next accf[b] phase
+        uint32_t xacc_par = 0;   // parity of the next xacc phase
         for (int J = 0; J < npanels; J++) {
             const int c0 = J * P, nk = c0 / BK, ncols = min(P, n - c0), nsb = ncols / PSB;
             const uint32_t acc = tl + (uint32_t)((J & 1) * P);
@@ -461,36 +490,53 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                                 make_float4(x[4 * q], x[4 * q + 1], x[4 * q + 2], x[4 * q + 3]);
                     }
                 }
-                // acc[tb] += x L[tb, sb]^T for the later sub-blocks; TMEM loads one
-                // sub-block ahead, stores unwaited until the next sub-block reads TMEM
+                // acc[:, later] += x_sb L[later, sb]^T for the later sub-blocks of the panel: one
+                // tcgen05 3xTF32 MMA group (M = 128 rows, N = the later columns, K = 16) issued by
+                // one epilogue thread into the panel's TMEM accumulator, operands staged in the
+                // XS area (SW64 K-major: A = the 128 rows' 16 solved values, B = rows of L_JJ)
+                if (e == 0) PANEL_T(J, 6 + 2 * sb);
                 if (sb + 1 < nsb) {
-                    float a[PSB], an[PSB];
-                    tmem_ld16_issue(acc + (sb + 1) * PSB, a);
-                    tmem_wait_ld(a);
-#pragma unroll 1
-                    for (int tb = sb + 1; tb < nsb; tb++) {
-                        if (tb + 1 < nsb) tmem_ld16_issue(acc + (tb + 1) * PSB, an);
+                    const int nb = (nsb - sb - 1) * PSB;   // later columns (a multiple of 16)
+                    {   // A: this row's values, split big / small
+                        const uint32_t ra = (uint32_t)e * 64u;
 #pragma unroll
-                        for (int c = 0; c < PSB; c++) {
-                            const float *lc = Lt + (sb * PSB + c) * LD + tb * PSB;
-#pragma unroll
-                            for (int q = 0; q < PSB / 4; q++) {
-                                const float4 l4 = *reinterpret_cast<const float4 *>(lc + 4 * q);
-                                a[4 * q + 0] = fmaf(x[c], l4.x, a[4 * q + 0]);
-                                a[4 * q + 1] = fmaf(x[c], l4.y, a[4 * q + 1]);
-                                a[4 * q + 2] = fmaf(x[c], l4.z, a[4 * q + 2]);
-                                a[4 * q + 3] = fmaf(x[c], l4.w, a[4 * q + 3]);
-                            }
-                        }
-                        tmem_st16_issue(acc + tb * PSB, a);
-                        if (tb + 1 < nsb) {
-                            tmem_wait_ld(an);
-#pragma unroll
-                            for (int i = 0; i < PSB; i++) a[i] = an[i];
+                        for (int q = 0; q < 4; q++) {
+                            const uint32_t off = ra + ((uint32_t)(q ^ ((e >> 1) & 3)) << 4);
+                            store_split(xs_ab, xs_as, off, make_float4(x[4 * q], x[4 * q + 1], x[4 * q + 2], x[4 * q + 3]));
                         }
                     }
-                    tmem_wait_st();
+                    if (e < nb) {   // B: row (sb+1)*16 + e of L_JJ, columns sb*16 .. +15 (from Lt)
+                        const float *lc = Lt + (sb * PSB) * LD + (sb + 1) * PSB + e;
+                        const uint32_t rb = (uint32_t)e * 64u;
+#pragma unroll
+                        for (int q = 0; q < 4; q++) {
+                            const float4 v = make_float4(lc[(4 * q) * LD], lc[(4 * q + 1) * LD], lc[(4 * q + 2) * LD],
+                                                         lc[(4 * q + 3) * LD]);
+                            store_split(xs_bb, xs_bs, rb + ((uint32_t)(q ^ ((e >> 1) & 3)) << 4), v);
+                        }
+                    }
+                    fence_proxy_async();
+                    tc_fence_before();
+                    bar_epi();
+                    if (e == 0) {
+                        tc_fence_after();
+                        const uint32_t idesc = make_idesc(BM, nb, false, false);
+                        const uint32_t d = tmem + (uint32_t)((J & 1) * P + (sb + 1) * PSB);
+                        const uint32_t ab = smem_u32(xs_ab), as = smem_u32(xs_as), bb = smem_u32(xs_bb), bs = smem_u32(xs_bs);
+#pragma unroll
+                        for (int kk = 0; kk < PSB / 8; kk++) {
+                            const uint32_t o = kk * 32;
+                            mma_tf32(d, desc_sw64(ab + o), desc_sw64(bb + o), idesc, 1u);
+                            mma_tf32(d, desc_sw64(ab + o), desc_sw64(bs + o), idesc, 1u);
+                            mma_tf32(d, desc_sw64(as + o), desc_sw64(bb + o), idesc, 1u);
+                        }
+                        mma_commit(xacc);
+                    }
+                    mbar_wait(xacc, xacc_par);
+                    xacc_par ^= 1u;
+                    tc_fence_after();
                 }
+                if (e == 0) PANEL_T(J, 7 + 2 * sb);
 #pragma unroll
                 for (int q = 0; q < 4; q++) bq[q] = bn[q];
             }
