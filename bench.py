@@ -702,6 +702,9 @@ def main():
             "host_us_per_task": {k: round((getattr(st1, "host_ns_" + k) - getattr(st0, "host_ns_" + k)) / 1e3 / max(1, len(log)), 3)
                                  for k in ("decide", "issue", "launch", "deps", "poll", "vevent", "flush")},
             "host_idle_loops_per_task": round((st1.host_idle_loops - st0.host_idle_loops) / max(1, len(log)), 2),
+            "host_us_per_group_launch": round((st1.host_ns_group_launch - st0.host_ns_group_launch) / 1e3 /
+                                              max(1, st1.group_launches - st0.group_launches), 2),
+            "group_launches_per_step": int((st1.group_launches - st0.group_launches) / args.steps),
             "host_loops_per_task": round((st1.host_loops - st0.host_loops) / max(1, len(log)), 2),
         }
         print(json.dumps(out))

@@ -300,6 +300,8 @@ typedef struct {
     int64_t host_ns_flush;    /* host time launching pending grouped launches from the loop */
     int64_t host_idle_loops;  /* drive-loop iterations that found nothing to do */
     int64_t device_released;  /* tasks made ready by the device dependence tracker (a3) */
+    int64_t host_ns_group_launch; /* host time inside grouped kernel launches */
+    int64_t group_launches;   /* grouped kernel launches issued */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 
