@@ -105,8 +105,10 @@ enum {
                              7 int8 slices under a power-of-two row scale (a cached "slice form",
                              like tc_3xf16's split form), the 28 slice products with i + j <= 8
                              accumulated exactly in int32 TMEM (one accumulator per diagonal),
-                             combined in fp64; MATMUL, GEMM_NT, SYRK, and TRSM as X = B inv(L)^T
-                             with the slice form of inv(L) (like tc_3xf16's R31); no POTRF */
+                             combined in fp64; MATMUL, GEMM_NT, SYRK; TRSM as X = B inv(L)^T
+                             with the slice form of inv(L) (like tc_3xf16's R31); POTRF
+                             recursive (DFMA diagonal blocks, DMMA panel trsm, Ozaki trailing
+                             updates on slice forms built inside the task) */
     VS_NUM_BUILTIN_VERSIONS = 7
 };
 
@@ -232,8 +234,8 @@ int vs_version_add(vs_rt rt, vs_type_id type, const char *name, uint32_t gpu_mas
  * set in version_mask (bit = VS_V_*).  Versions each type actually gets:
  *   VS_F32: SIMT_F32, TC_3XTF32, F64IN_F32IO for all five types; TC_3XF16 for MATMUL,
  *           GEMM_NT, SYRK and TRSM (by inverse, R31) — not POTRF.
- *   VS_F64: DFMA_F64, DMMA_F64 for all five types; OZ_I8_F64 for MATMUL, GEMM_NT, SYRK and
- *           TRSM (by inverse) — not POTRF.
+ *   VS_F64: DFMA_F64, DMMA_F64 and OZ_I8_F64 for all five types (OZ_I8_F64: TRSM by inverse,
+ *           POTRF recursive with Ozaki-scheme trailing updates).
  * out_types[VS_T_*] receives the type ids.  Version INDICES are per type: inside each type
  * the kept versions are numbered 0, 1, ... in increasing VS_V_* order, skipping those the type
  * does not get, so the same index may name different versions in different types (e.g. with

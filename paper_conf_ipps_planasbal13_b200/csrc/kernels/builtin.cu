@@ -95,6 +95,39 @@ struct DmmaEngine {
         return blocked_trsm<Tin, Tp, DmmaEngine>(rows, n, L, ldl, X, ldx, s, ctx);
     }
 };
+// oz_i8_f64 POTRF (recursive, like the DFMA / DMMA versions): the trailing updates are Ozaki-
+// scheme tcgen05 kind::i8 GEMMs on slice forms built per call in stream-ordered scratch; the
+// panel trsm is the blocked DMMA substitution, the diagonal blocks the DFMA register kernel.
+struct OzEngine {
+    using Tp = double;
+    template <bool NT, bool NEG, bool LOWER>
+    static int gemm(int M, int N, int K, const double *A, int lda, const double *B, int ldb, double *C, int ldc,
+                    cudaStream_t s, const TaskCtx &ctx)
+    {
+        static_assert(NT && NEG, "potrf_rec only needs C -= A B^T");
+        if (M <= 0 || N <= 0 || K <= 0) return 0;
+        // the small updates near the recursion's leaves stay on DMMA (slice forms need K % 64,
+        // N % 64, and do not pay off below 128)
+        if (K % 64 || N % oz::BN || M < 128 || N < 128 || K < 128 || (LOWER && M != N))
+            return DmmaEngine<double>::template gemm<NT, NEG, LOWER>(M, N, K, A, lda, B, ldb, C, ldc, s, ctx);
+        const size_t fa = (oz::form_bytes(M, K) + 255) / 256 * 256;
+        const size_t fb = LOWER ? 0 : (oz::form_bytes(N, K) + 255) / 256 * 256;
+        void *buf = nullptr;
+        if (cudaMallocAsync(&buf, fa + fb, s) != cudaSuccess) return -1;
+        uint8_t *pa = (uint8_t *)buf, *pb = LOWER ? pa : pa + fa;
+        int r = oz::make_slices(A, M, K, lda, 1, 128, pa, s, true);
+        if (!r && !LOWER) r = oz::make_slices(B, N, K, ldb, 1, 64, pb, s, true);
+        if (!r) r = LOWER ? oz::oz_gemm<true, true, 128>(M, N, K, pa, pb, C, ldc, s, false, ctx)
+                          : oz::oz_gemm<true, false, 64>(M, N, K, pa, pb, C, ldc, s, false, ctx);
+        cudaFreeAsync(buf, s);
+        return r;
+    }
+    static int trsm(int rows, int n, const double *L, int ldl, double *X, int ldx, cudaStream_t s, const TaskCtx &ctx)
+    {
+        return DmmaEngine<double>::trsm(rows, n, L, ldl, X, ldx, s, ctx);
+    }
+};
+
 struct TcEngine {
     using Tp = float;
     template <bool NT, bool NEG, bool LOWER>
@@ -171,7 +204,6 @@ bool builtin_supported(int type, int version, int b)
     if (type < 0 || type >= VS_NUM_BUILTIN_TYPES) return false;
     if (version < 0 || version >= VS_NUM_BUILTIN_VERSIONS) return false;
     if (version == VS_V_TC_3XF16 && type == VS_T_POTRF) return false;
-    if (version == VS_V_OZ_I8_F64 && type == VS_T_POTRF) return false;
     if (b && (b % 64 != 0 || b < 64 || b > 4096)) return false;
     return true;
 }
@@ -276,9 +308,10 @@ int group_launch(TaskGroup *g, cudaStream_t s) { return tcf::tcf_group_launch(g-
 
 namespace {
 // oz_i8_f64: p[np + i] holds the slice forms of the in-operands (builtin_operand_form)
-int run_oz(int type, int b, void *const *p, cudaStream_t s, const TaskCtx &ctx)
+int run_oz(int type, int b, void *const *p, int *info, cudaStream_t s, const TaskCtx &ctx)
 {
     switch (type) {
+    case VS_T_POTRF: return potrf_rec<double, OzEngine>((double *)p[0], b, b, 0, info, s, ctx);   // A = L L^T
     case VS_T_MATMUL: return oz::oz_gemm<false, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, false, ctx);   // C += A B
     case VS_T_GEMM_NT: return oz::oz_gemm<true, false, 64>(b, b, b, p[3], p[4], (double *)p[2], b, s, false, ctx);  // C -= A B^T
     case VS_T_SYRK: return oz::oz_gemm<true, true, 128>(b, b, b, p[2], p[2], (double *)p[1], b, s, false, ctx);   // C -= A A^T
@@ -348,7 +381,7 @@ int launch_builtin(int type, int version, int b, void *const *p, int *info, cuda
     case VS_V_DFMA_F64: return run_family<double, SimtEngine<double, double>>(type, b, p, info, s, ctx);
     case VS_V_DMMA_F64: return run_family<double, DmmaEngine<double>>(type, b, p, info, s, ctx);
     case VS_V_TC_3XF16: return run_f16(type, b, p, s, ctx);
-    case VS_V_OZ_I8_F64: return run_oz(type, b, p, s, ctx);
+    case VS_V_OZ_I8_F64: return run_oz(type, b, p, info, s, ctx);
     }
     return -1;
 }

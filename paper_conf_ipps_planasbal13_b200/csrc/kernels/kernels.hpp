@@ -15,6 +15,15 @@ inline std::atomic<long long> &launch_counter()
     return c;
 }
 inline void count_launch() { launch_counter().fetch_add(1, std::memory_order_relaxed); }
+// Kernels a version launches for itself that carry no execution record (e.g. the operand
+// forms oz_i8_f64's POTRF builds for its trailing updates): reported in the launch count, but
+// not part of a task's kernel count (the completion of its record-carrying kernels).
+inline std::atomic<long long> &aux_launch_counter()
+{
+    static std::atomic<long long> c{0};
+    return c;
+}
+inline void count_launch_aux() { aux_launch_counter().fetch_add(1, std::memory_order_relaxed); }
 
 // Device dependence tracker (a3): in-degrees and CSR successor lists of
 // the tasks of one drive, in device memory of the runtime's GPU, built by the runtime at the

@@ -333,14 +333,18 @@ __global__ void __launch_bounds__(NTHREADS, 1)
 
 // ---------------------------------------------------------------- host launchers
 // Slice form of an R x K operand: element (r, k) = X[r * sr + k * sk].
-inline int make_slices(const double *X, int R, int K, int64_t sr, int64_t sk, int G, void *out, cudaStream_t s)
+// aux: launched inside a version's task (no execution record; count_launch_aux)
+inline int make_slices(const double *X, int R, int K, int64_t sr, int64_t sk, int G, void *out, cudaStream_t s,
+                       bool aux = false)
 {
     if (R <= 0 || K <= 0 || K % 64) return -1;
     const int Rp = rows_padded(R);
-    count_launch();
+    if (aux) count_launch_aux();
+    else count_launch();
     if (sk == 1) oz_scale_kernel<<<(Rp + 7) / 8, 256, 0, s>>>(X, R, K, sr, sk, (uint8_t *)out);
     else oz_scale_kernel<<<(Rp + 255) / 256, 256, 0, s>>>(X, R, K, sr, sk, (uint8_t *)out);
-    count_launch();
+    if (aux) count_launch_aux();
+    else count_launch();
     const int64_t n = (int64_t)Rp * (K / 16);
     oz_slice_kernel<<<(unsigned)((n + 255) / 256), 256, 0, s>>>(X, R, K, sr, sk, G, (uint8_t *)out);
     return 0;

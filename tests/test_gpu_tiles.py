@@ -192,7 +192,7 @@ def test_trsm_tile(gpu, version, b):
     assert oracle.relF(X, oracle.trsm(L, X0)) <= _gate(version)
 
 
-@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS + [vs.VS_V_OZ_I8_F64])
 @pytest.mark.parametrize("b", [64, 128, 192, 512, 1024])
 def test_potrf_tile(gpu, version, b):
     torch = _torch()
@@ -211,7 +211,7 @@ def test_potrf_tile(gpu, version, b):
     assert np.all(L[np.triu_indices(b, 1)] == 777.0)                  # R7
 
 
-@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS)
+@pytest.mark.parametrize("version", F32_VERSIONS + F64_VERSIONS + [vs.VS_V_OZ_I8_F64])
 def test_potrf_integer_L0_exact_and_info(gpu, version):
     torch = _torch()
     dt = _dt(version)
