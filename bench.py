@@ -482,7 +482,9 @@ def run_reference(args, rank, world):
     gf = f / t / 1e9
     s0 = samples[0]
     sample = ("per step: oracle fp64 matmul rows 0..%d of C=A*B at N=16384 + oracle unblocked Cholesky of the "
-              "leading %dx%d block of the cfg4 SPD matrix" % (s0["rows"] - 1, s0["k"], s0["k"]))
+              "leading %dx%d block of the cfg4 SPD matrix; value = the sample's flops / its time, not extrapolated "
+              "(an upper bound for the full workload: the %dx%d factor is cache-resident)" % (
+                  s0["rows"] - 1, s0["k"], s0["k"], s0["k"], s0["k"]))
     out = {"metric": "tiled matmul & Cholesky GFLOP/s", "value": round(gf, 3), "unit": "GFLOP/s", "impl": "reference",
            "n_gpus": args.gpus, "steps": args.steps, "warmup": args.warmup,
            "ms_per_step": round(1e3 * t / len(samples), 2), "higher_is_better": True,
@@ -670,8 +672,10 @@ def main():
         cpu = {"value": round((s["f_mm"] + s["f_ch"]) / (s["t_mm"] + s["t_ch"]) / 1e9, 3), "unit": "GFLOP/s",
                "cores": s["cores"], "kind": "oracle",
                "sample": "oracle fp64 matmul rows 0..%d of C=A*B at N=%d (%.1f s) + oracle unblocked Cholesky of the "
-                         "leading %dx%d block of the cfg4 SPD matrix (%.1f s)" % (
-                             s["rows"] - 1, MM_N, s["t_mm"], s["k"], s["k"], s["t_ch"])}
+                         "leading %dx%d block of the cfg4 SPD matrix (%.1f s); value = the sample's flops / its time, "
+                         "not extrapolated; an upper bound for the full workload (the %dx%d factor is cache-resident, "
+                         "the N=%d one is not)" % (
+                             s["rows"] - 1, MM_N, s["t_mm"], s["k"], s["k"], s["t_ch"], s["k"], s["k"], CH_N)}
 
     if rank == 0:
         out = {
