@@ -44,8 +44,11 @@ SEED_MM, SEED_CH = 3, 4
 # no cross-stream waits, so no stream is blocked at its head), NEXT-4 bottom-level priority
 # with a real queue cap of 1 grouped launch (8 tasks) per worker, grouped launches of up to 8
 # tc_3xf16 tasks held up to 200 us while their stream still runs a kernel (group_hold),
-# critical-path tasks on their own greatest-priority streams
-RT_DEFAULTS = dict(lam=3, slots=12, priority=2, qdepth=1, group=8, mode="ready", hold=1, group_us=200)
+# critical-path tasks on their own greatest-priority streams, dependences released on the device
+# (a3: in-degree counters + CSR successors on the GPU, ready ring; measured within 0.5 % of the
+# host release; VS_BENCH_DEVICE_RELEASE=0 switches back)
+RT_DEFAULTS = dict(lam=3, slots=12, priority=2, qdepth=1, group=8, mode="ready", hold=1, group_us=200,
+                   device_release=int(os.environ.get("VS_BENCH_DEVICE_RELEASE", "1")))
 F32_VERSIONS_MASK = 0b100111  # simt_f32 | tc_3xtf32 | f64in_f32io | tc_3xf16 (gemm-type tasks)
 MM_FLOPS = lambda n: 2.0 * n ** 3            # noqa: E731  (reading R6)
 CH_FLOPS = lambda n: n ** 3 / 3.0            # noqa: E731
@@ -56,7 +59,7 @@ def bench_config(vs, **over):
     d = RT_DEFAULTS
     kw = dict(lam=d["lam"], slots_per_gpu=d["slots"], priority=d["priority"], queue_depth=d["qdepth"],
               group_tasks=d["group"], mode=1 if d["mode"] == "ready" else 0, group_hold=d["hold"],
-              group_wait_us=d["group_us"])
+              group_wait_us=d["group_us"], device_release=d["device_release"])
     kw.update(over)
     return vs.vs_config_default(**kw)
 
@@ -562,7 +565,8 @@ def main():
     mode = 1 if args.mode == "ready" else 0          # VS_MODE_READY / VS_MODE_RUNAHEAD
     cfg = vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, device_base=rank_device(local, ndev),
                                replay=1 if args.replay else 0, priority=prio, lookahead=look, queue_depth=qdepth,
-                               group_tasks=args.group, mode=mode, group_hold=args.hold, group_wait_us=args.group_us)
+                               group_tasks=args.group, mode=mode, group_hold=args.hold, group_wait_us=args.group_us,
+                               device_release=RT_DEFAULTS["device_release"])
     rt = vs.Runtime(cfg)
     if world > 1:
         shm = gather("/vsched_%d_%d" % (os.getpid(), int(time.time())) if rank == 0 else None)[0]
@@ -634,7 +638,8 @@ def main():
     if not args.no_e2e and world == 1:
         rt2 = vs.Runtime(vs.vs_config_default(lam=args.lam, slots_per_gpu=args.slots, priority=prio, lookahead=look,
                                               queue_depth=qdepth, group_tasks=args.group, mode=mode,
-                                              group_hold=args.hold, group_wait_us=args.group_us))
+                                              group_hold=args.hold, group_wait_us=args.group_us,
+                                              device_release=RT_DEFAULTS["device_release"]))
         wl2 = Workload(rt2, mm_n, mm_b, ch_n, ch_b, host=True, with_mm=with_mm, with_ch=with_ch)
         wl2.step()     # warm-up incl. learning
         tsum, h2d, d2h = 0.0, 0, 0
@@ -698,7 +703,8 @@ def main():
             "device completion words (stream memops)" if st1.tracker == 1 else "host (completion ring + cuda events)",
             "runtime_options": {"lookahead": look, "priority": prio, "queue_depth": qdepth, "group_tasks": args.group,
                                 "group_hold": args.hold, "group_wait_us": args.group_us,
-                                "mode": args.mode, "cuda_device_max_connections": os.environ.get("CUDA_DEVICE_MAX_CONNECTIONS")},
+                                "mode": args.mode, "device_release": RT_DEFAULTS["device_release"],
+                                "cuda_device_max_connections": os.environ.get("CUDA_DEVICE_MAX_CONNECTIONS")},
             "tasks_per_step": int((st1.tasks_completed - st0.tasks_completed) / args.steps),
             "version_counts": version_counts,
             "operand_forms_per_step": int((st1.forms_built - st0.forms_built) / args.steps),
