@@ -32,6 +32,7 @@
 #include "tc_gemm.cuh"
 #include "tc_f16.cuh"
 #include "tc_oz.cuh"
+#include "tc_inv.cuh"
 #include "tc_panel.cuh"
 
 #include "vsched.h"
@@ -262,13 +263,14 @@ int make_form(int form, int b, const void *src, void *dst, cudaStream_t s)
     if (form == FORM_SPLIT_ROWS) return tcf::split_rows((const float *)src, b, b, b, dst, s);
     if (form == FORM_SPLIT_COLS) return tcf::split_cols((const float *)src, b, b, b, dst, s);
     if (form == FORM_INV_L) {
-        // X = I L^{-T} by the substitution kernel of tc_3xtf32 (tc_panel; measured 258 us at
-        // b = 1024 against 719 us for the sub-tile DAG of blk_chol.cuh), then the row split
-        // form of X^T = inv(L): reading R31 (TRSM of tc_3xf16 multiplies by it)
+        // X = L^{-T} by recursive doubling on the 3xTF32 kernels (tc_inv.cuh; the whole-tile
+        // substitution of tc_panel took 258 us at b = 1024, the sub-tile DAG of blk_chol.cuh
+        // 719 us), then the row split form of X^T = inv(L): reading R31 (TRSM of tc_3xf16
+        // multiplies by it).  The split area is the recursion's scratch until split_cols.
         float *X = (float *)((uint8_t *)dst + (tcf::split_bytes(b, b) + 255) / 256 * 256);
         count_launch();
         tcf::eye_kernel<<<148, 256, 0, s>>>(X, b);
-        if (tc::tc_trsm(b, b, (const float *)src, b, X, b, s)) return -1;
+        if (tc::tc_inv_lt(b, (const float *)src, b, X, b, (float *)dst, s)) return -1;
         return tcf::split_cols(X, b, b, b, dst, s);
     }
     return -1;

@@ -688,8 +688,14 @@ inline int tcf_group_launch(TcfGroup &g, cudaStream_t s)
 
 __global__ void eye_kernel(float *X, int n)
 {
-    for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < (int64_t)n * n; i += (int64_t)gridDim.x * blockDim.x)
-        X[i] = (i / n == i % n) ? 1.f : 0.f;
+    // n % 4 == 0: float4 stores, rows strided over the grid
+    const int nq = n / 4;
+    for (int r = blockIdx.x; r < n; r += gridDim.x)
+        for (int q = threadIdx.x; q < nq; q += blockDim.x) {
+            const bool d = (r >> 2) == q;
+            const float4 v = make_float4(d && (r & 3) == 0, d && (r & 3) == 1, d && (r & 3) == 2, d && (r & 3) == 3);
+            reinterpret_cast<float4 *>(X + (int64_t)r * n)[q] = v;
+        }
 }
 
 // C (M x N, ldc) += s * A * B'^T with A, B' in split form (K a multiple of 32): one task.

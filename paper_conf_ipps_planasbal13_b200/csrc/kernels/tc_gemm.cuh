@@ -187,12 +187,24 @@ __device__ __forceinline__ void nn_unit(int t, int p, int &kq, int &nq)
     nq = (lane & 1) | (((lane >> 3) & 3) << 1) | ((idx % NG) << 3);
 }
 
-template <int BN, bool NT, bool NEG, bool LOWER>
+// a batch of equally shaped products, one per blockIdx.z (element strides; the inverse form of
+// tc_inv.cuh), and beta0: C_in taken as zero (C is written, not read)
+struct GemmBatch {
+    int64_t a = 0, b = 0, c = 0;
+    int beta0 = 0;
+};
+
+template <int BN, bool NT, bool NEG, bool LOWER, bool BATCH = false>
 __global__ void __launch_bounds__(NTHREADS, 1)
 tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const float *__restrict__ B, int ldb,
-               float *__restrict__ C, int ldc, TaskCtx ctx)
+               float *__restrict__ C, int ldc, GemmBatch bt, TaskCtx ctx)
 {
     ctx_begin(ctx);
+    if (BATCH) {   // a compile-time switch: the batch fields cost the tile kernel a register
+        A += blockIdx.z * bt.a;
+        B += blockIdx.z * bt.b;
+        C += blockIdx.z * bt.c;
+    }
     using G = Cfg<BN>;
     constexpr int STAGES = G::STAGES;
     extern __shared__ uint8_t smem_raw[];
@@ -306,24 +318,43 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
             const float *crow = C + (int64_t)erow * ldc + n0 + col0;
 #pragma unroll
             for (int j = 0; j < 8; j++) {
-                const float4 x = (erow < M && n0 + col0 + 4 * j < N) ? *reinterpret_cast<const float4 *>(crow + 4 * j) : z4;
+                const float4 x = (!(BATCH && bt.beta0) && erow < M && n0 + col0 + 4 * j < N) ? *reinterpret_cast<const float4 *>(crow + 4 * j) : z4;
                 v[4 * j] = x.x; v[4 * j + 1] = x.y; v[4 * j + 2] = x.z; v[4 * j + 3] = x.w;
             }
             tmem_st32(tmem + ((uint32_t)(eq * 32) << 16) + (uint32_t)(BN + col0), v);
         };
-        // two k-blocks of loads in flight (register double buffer, loop unrolled by 2)
-        float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
-        load(ra0, rb0, 0);
-        if (nk > 1) load(ra1, rb1, 1);
+        // D k-blocks of loads in flight (register buffers, loop unrolled by D): 2 for the wide
+        // tile, 3 for BN = 128 (its small grids are latency-bound: the inverse form)
         int staged = 0;
-        for (int kb = 0; kb < nk; kb += 2) {
-            produce(ra0, rb0, kb);
-            if (kb + 2 < nk) load(ra0, rb0, kb + 2);
-            if (staged < NCH) stage_c(staged++);
-            if (kb + 1 < nk) {
-                produce(ra1, rb1, kb + 1);
-                if (kb + 3 < nk) load(ra1, rb1, kb + 3);
+        if constexpr (BN > 128) {
+            float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
+            load(ra0, rb0, 0);
+            if (nk > 1) load(ra1, rb1, 1);
+            for (int kb = 0; kb < nk; kb += 2) {
+                produce(ra0, rb0, kb);
+                if (kb + 2 < nk) load(ra0, rb0, kb + 2);
                 if (staged < NCH) stage_c(staged++);
+                if (kb + 1 < nk) {
+                    produce(ra1, rb1, kb + 1);
+                    if (kb + 3 < nk) load(ra1, rb1, kb + 3);
+                    if (staged < NCH) stage_c(staged++);
+                }
+            }
+        } else {
+            constexpr int D = 3;
+            float4 ra[D][APER], rb[D][BPER];
+#pragma unroll
+            for (int d = 0; d < D; d++)
+                if (d < nk) load(ra[d], rb[d], d);
+            for (int kb = 0; kb < nk; kb += D) {
+#pragma unroll
+                for (int d = 0; d < D; d++) {
+                    if (kb + d < nk) {
+                        produce(ra[d], rb[d], kb + d);
+                        if (kb + d + D < nk) load(ra[d], rb[d], kb + d + D);
+                        if (staged < NCH) stage_c(staged++);
+                    }
+                }
             }
         }
         while (staged < NCH) stage_c(staged++);
@@ -399,13 +430,14 @@ tc_gemm_kernel(int M, int N, int K, const float *__restrict__ A, int lda, const 
 }
 
 // Host launcher: K multiple of 32; lda/ldb/ldc multiples of 4 and 16-byte aligned bases.
-template <bool NT, bool NEG, bool LOWER, int BN = 256>
+// BATCH: count products along blockIdx.z with the element strides of bt (bt.beta0: C_in = 0)
+template <bool NT, bool NEG, bool LOWER, int BN = 256, bool BATCH = false>
 inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B, int ldb, float *C, int ldc,
-                   cudaStream_t s, const TaskCtx &ctx = TaskCtx())
+                   cudaStream_t s, const TaskCtx &ctx = TaskCtx(), const GemmBatch &bt = GemmBatch(), int count = 1)
 {
     if (M <= 0 || N <= 0) return 0;
-    if (K % BK) return -1;
-    auto kern = tc_gemm_kernel<BN, NT, NEG, LOWER>;
+    if (K % BK || (!BATCH && (count != 1 || bt.beta0))) return -1;
+    auto kern = tc_gemm_kernel<BN, NT, NEG, LOWER, BATCH>;
     constexpr int smem = Cfg<BN>::SMEM;
     static bool attr[64] = {};
     int dev = 0;
@@ -414,7 +446,7 @@ inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B,
         cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
         attr[dev & 63] = true;
     }
-    dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM);
+    dim3 grid((N + BN - 1) / BN, (M + BM - 1) / BM, count);
     // The tensor core's fp32 accumulation does not round to nearest: its error grows linearly
     // with the accumulated K (measured relF of a b x b MATMUL: 7.2e-6 at K = 1024, 1.4e-5 at 2048,
     // 2.9e-5 at 4096).  K is therefore cut into chunks of at most kKChunk, one launch each; every
@@ -423,9 +455,11 @@ inline int tc_gemm(int M, int N, int K, const float *A, int lda, const float *B,
     const TaskCtx c = ctx_for(ctx, kern, NTHREADS, smem);
     for (int k0 = 0; k0 < K; k0 += kKChunk) {
         const int kc = K - k0 < kKChunk ? K - k0 : kKChunk;
+        GemmBatch bc = bt;
+        if (k0 > 0) bc.beta0 = 0;   // later chunks accumulate onto the first one's result
         count_launch();
         kern<<<grid, NTHREADS, smem, s>>>(M, N, kc, A + k0, lda, B + (NT ? (int64_t)k0 : (int64_t)k0 * ldb), ldb, C, ldc,
-                                          c);
+                                          bc, c);
     }
     return 0;
 }

@@ -193,9 +193,11 @@ __device__ __forceinline__ uint64_t desc_sw64(uint32_t saddr)
 template <bool POTRF>
 __global__ void __launch_bounds__(PTHREADS, 1)
 tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int k_base, int *info,
-                unsigned long long launch_id, int overlap, TaskCtx ctx)
+                unsigned long long launch_id, int overlap, int64_t lbs, int64_t xbs, TaskCtx ctx)
 {
     ctx_begin(ctx);
+    L += blockIdx.y * lbs;   // TRSM batch (tc_trsm_batched): independent problems along y
+    X += blockIdx.y * xbs;
     using G = PanelCfg;
     constexpr int P = PNL, STAGES = G::STAGES, LD = G::LD, NP = G::NP;
     extern __shared__ uint8_t smem_raw[];
@@ -594,7 +596,20 @@ inline int tc_trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, 
     panel_attr<false>();
     count_launch();
     tc_panel_kernel<false><<<(rows + BM - 1) / BM, PTHREADS, PanelCfg::SMEM, s>>>(rows, n, L, ldl, X, ldx, 0, nullptr,
-                                                                                  0ull, panel_overlap(), ctx);
+                                                                                  0ull, panel_overlap(), 0, 0, ctx);
+    return 0;
+}
+
+// count independent X_i <- X_i L_i^{-T} (X_i = X + i xbs, L_i = L + i lbs), one launch.
+inline int tc_trsm_batched(int count, int rows, int n, const float *L, int ldl, int64_t lbs, float *X, int ldx,
+                           int64_t xbs, cudaStream_t s)
+{
+    if (rows <= 0 || n <= 0 || count <= 0) return 0;
+    if (n % 64) return -1;
+    panel_attr<false>();
+    count_launch();
+    tc_panel_kernel<false><<<dim3((rows + BM - 1) / BM, count), PTHREADS, PanelCfg::SMEM, s>>>(
+        rows, n, L, ldl, X, ldx, 0, nullptr, 0ull, panel_overlap(), lbs, xbs, TaskCtx());
     return 0;
 }
 
@@ -608,7 +623,7 @@ inline int tc_potrf(int n, float *A, int lda, int k_base, int *info, cudaStream_
     panel_attr<true>();
     count_launch();
     tc_panel_kernel<true><<<(n + BM - 1) / BM, PTHREADS, PanelCfg::SMEM, s>>>(n, n, A, lda, A, lda, k_base, info, id,
-                                                                             panel_overlap(), ctx);
+                                                                             panel_overlap(), 0, 0, ctx);
     return 0;
 }
 

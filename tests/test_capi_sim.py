@@ -169,6 +169,39 @@ def test_table_i_and_new_group(tmp_path):
         assert "task1 %d task1-v1 45000000 80" % (3 * MB) in out.read_text()   # untouched group entry
 
 
+def test_weighted_bottom_level_matches_model(tmp_path):
+    """R29 / R38 through the C ABI: learned means (warm-start table) weight the bottom levels;
+    the same graph as tests/test_sched_fixtures.py::test_weighted_bottom_level_uses_learned_means,
+    C++ log = model log."""
+    p = tmp_path / "w.txt"
+    p.write_text("A 8 v 100 1\nB 8 v 10 1\n")
+    rt = _sim(1, 1, 1, priority=2, queue_depth=1)
+    ta = rt.vs_type_create("A", [vs.VS_INOUT])
+    rt.vs_version_add(ta, "v", ALL)
+    tb = rt.vs_type_create("B", [vs.VS_INOUT])
+    rt.vs_version_add(tb, "v", ALL)
+    rt.vs_table_load(str(p))
+    a = rt.vs_data_register(_fake_ptr(0, 8), 0, 8)
+    b = rt.vs_data_register(_fake_ptr(1, 8), 0, 8)
+    for t, d, n in ((ta, a, 2), (tb, b, 3)):
+        for _ in range(n):
+            rt.vs_submit(t, [d])
+    rt.vs_replay_set(ta, 8, 0, 100)
+    rt.vs_replay_set(tb, 8, 0, 10)
+    rt.vs_wait_all()
+    got = rt.vs_decision_log()
+    m = SchedModel(1, 1, 1, priority=2, qdepth=1)
+    ma, mb = m.add_type("A", [("v", ALL)]), m.add_type("B", [("v", ALL)])
+    da, db = m.add_data(8), m.add_data(8)
+    for t, d, n in ((ma, da, 2), (mb, db, 3)):
+        for _ in range(n):
+            m.submit(t, [(d, "inout")])
+    m.load_table([(ma, 8, [(100, 1)]), (mb, 8, [(10, 1)])])
+    ref = m.simulate(lambda ty, nb, v: 100 if ty == ma else 10)
+    assert [r[:6] for r in got] == [r[:6] for r in ref]
+    assert [(r[0], r[3]) for r in got] == [(0, 0), (1, 100), (2, 200), (3, 210), (4, 220)]
+
+
 def test_fig5_earliest_executor_masks():
     # Fig 5: version "fast" runs only on gpu 3 (worker 3), "slow" only on gpu 2.
     rt = _sim(4, 1, 1)

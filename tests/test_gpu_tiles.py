@@ -182,7 +182,7 @@ def test_oz_i8_f64_row_scales_and_componentwise_bound(gpu, ttype):
 
 # ------------------------------------------------------------------ trsm / potrf
 @pytest.mark.parametrize("version", F32_VERSIONS + [vs.VS_V_TC_3XF16] + F64_VERSIONS + [vs.VS_V_OZ_I8_F64])
-@pytest.mark.parametrize("b", [64, 128, 192, 512, 1024])
+@pytest.mark.parametrize("b", [64, 128, 192, 320, 512, 1024])   # 192, 320: ragged inverse levels (R31)
 def test_trsm_tile(gpu, version, b):
     dt = _dt(version)
     Lfull, _ = oracle.cholesky(vsgen.spd(500 + b, b, np.float64))
@@ -246,6 +246,23 @@ def test_max_tile_4096_sampled_rows(gpu, version):
     (_, _, G) = _run(vs.VS_T_GEMM_NT, version, b, [A, B, C0])
     ref = oracle.matmul(-A[rows], np.ascontiguousarray(B.T), C0[rows])   # C0 - A B^T (negation exact)
     assert oracle.relF(G[rows], ref) <= 1e-5
+
+
+@pytest.mark.parametrize("b", [2048, 4096])
+def test_trsm_inverse_large(gpu, b):
+    # tc_3xf16's TRSM multiplies by the inv(L) form (R31), built by recursive doubling up to
+    # h = b / 2 (K = 2048 at b = 4096 runs in two accumulation chunks); L a well-conditioned
+    # lower triangle (unit-scale entries, diagonal b).  b = 2048: the whole tile against the
+    # oracle's substitution; b = 4096: sampled rows at block boundaries through the residual
+    # X L^T - B (the oracle's square-only trsm would take minutes there)
+    L = (np.tril(vsgen.uniform(810 + b, b, b, np.float64)) + b * np.eye(b)).astype(np.float32)
+    X0 = vsgen.uniform(811 + b, b, b)
+    (_, X) = _run(vs.VS_T_TRSM, vs.VS_V_TC_3XF16, b, [L, X0])
+    if b == 2048:
+        assert oracle.relF(X, oracle.trsm(L, X0)) <= 1e-5
+    else:
+        rows = [0, 63, 64, 1023, 1024, 2047, 2048, b - 1]
+        assert oracle.relF(oracle.matmul(X[rows], np.ascontiguousarray(L.T)), X0[rows]) <= 1e-5
 
 
 @pytest.mark.parametrize("b", [0, 32, 96, 8192])

@@ -12,7 +12,7 @@ C++ = model).  Each one is chosen so that a plausible misreading fails it:
 * NEXT-1 locality-aware earliest executor (L978-984): EFT + bytes not valid on the worker's
   GPU / bandwidth (1 GB/s = 1 byte/ns, integer division), validity updated in decision order
   (reads replicate, writes own);
-* NEXT-4 bottom-level priority + queue depth (R29);
+* NEXT-4 bottom-level priority + queue depth (R29), critical path first (R38);
 * the paper-literal "rr" learning variant (R12) against the default hold policy.
 """
 from oracle.sched_model import SchedModel
@@ -183,14 +183,76 @@ def test_bottom_levels():
     assert _prio_model(2, 1).bottom_levels() == [1, 3, 2, 1, 2, 1]
 
 
+def test_slacks():
+    # R38: top levels [1, 1, 2, 3, 1, 2], longest path L = 3 (t1 -> t2 -> t3); slack = L - (tl +
+    # bl - 1): t0 3 - 1 = 2, the chain 0, t4 / t5 3 - 2 = 1 (an exclusive "< 1" or a missing -1
+    # would change the critical set)
+    assert _prio_model(2, 1).slacks() == [2, 0, 0, 0, 1, 1]
+
+
 def test_bottom_level_order_with_queue_depth_1():
-    """Ready at 0: t0 (bl 1), t1 (bl 3), t4 (bl 2).  Depth 1: one task per worker at a time, the
-    rest stay in the ready heap (largest bl, then id).
-      0: t1.  10: t2 (bl 2) ties t4 (bl 2) -> lower id t2.  20: t4 (t3, t0 have bl 1).
-      30: t0, t3, t5 all bl 1 -> ids in order: t0 at 30, t3 at 40, t5 at 50."""
+    """Ready at 0: t0 (bl 1, slack 2), t1 (bl 3), t4 (bl 2).  Depth 1: one task per worker at a
+    time, the rest stay in the ready heap: slack <= 1 first (R38), then largest bl, then id.
+      0: t1.  10: t2 (bl 2) ties t4 (bl 2) -> lower id t2.  20: t4 (bl 2).
+      30: t0, t3, t5 all bl 1, t0 off the critical path -> t3 at 30, t5 at 40, t0 at 50
+      (bottom level alone would run t0 at 30)."""
     log = _prio_model(2, 1).simulate(lambda ty, nb, v: 10)
-    assert [(r[0], r[3], r[4]) for r in log] == [(1, 0, 0), (2, 10, 10), (4, 20, 20), (0, 30, 30),
-                                                (3, 40, 40), (5, 50, 50)]
+    assert [(r[0], r[3], r[4]) for r in log] == [(1, 0, 0), (2, 10, 10), (4, 20, 20), (3, 30, 30),
+                                                (5, 40, 40), (0, 50, 50)]
+
+
+def test_weighted_bottom_level_uses_learned_means():
+    """R29: types A (learned mean 100 ns) and B (10 ns); chain a0 -> a1 (t0, t1) and chain
+    b0 -> b1 -> b2 (t2, t3, t4); one worker, depth 1.  Weighted bottom levels: a0 = 200, a1 =
+    100, b0 = 30, b1 = 20, b2 = 10 (unit levels would be 2, 1, 3, 2, 1).  Slack (unit): L = 3,
+    every task <= 1, so all are on the critical path and the weighted level decides:
+      0: a0 (200 > 30), runs 0-100.  100: a1 (100) before b0 (30), runs 100-200.  200: b0,
+      210: b1, 220: b2.  (By unit levels b0 would go first, at 0.)  A task of an unlearned
+    group weighs 1000 ns."""
+    m = SchedModel(1, 1, 1, priority=2, qdepth=1)
+    ta = m.add_type("A", [("v", ALL)])
+    tb = m.add_type("B", [("v", ALL)])
+    a, b = m.add_data(8), m.add_data(8)
+    for _ in range(2):
+        m.submit(ta, [(a, "inout")])
+    for _ in range(3):
+        m.submit(tb, [(b, "inout")])
+    m.load_table([(ta, 8, [(100, 1)]), (tb, 8, [(10, 1)])])
+    assert m.weighted_bottom_levels() == [200, 100, 30, 20, 10]
+    log = m.simulate(lambda ty, nb, v: 100 if ty == ta else 10)
+    assert [(r[0], r[3]) for r in log] == [(0, 0), (1, 100), (2, 200), (3, 210), (4, 220)]
+    m2 = SchedModel(1, 1, 1, priority=2, qdepth=1)
+    t2 = m2.add_type("A", [("v", ALL)])
+    d = m2.add_data(8)
+    for _ in range(2):
+        m2.submit(t2, [(d, "inout")])
+    assert m2.weighted_bottom_levels() == [2000, 1000]
+
+
+def _crit_model():
+    """Chain a0 -> ... -> a5 (the critical path, L = 6); chain b0 -> b1 -> b2 -> b3 (bl 4, slack
+    2); one worker, depth 1, 10 ns each."""
+    m = SchedModel(1, 1, 1, priority=2, qdepth=1)
+    t = m.add_type("T", [("v", ALL)])
+    a, b = m.add_data(8), m.add_data(8)
+    for _ in range(6):
+        m.submit(t, [(a, "inout")])                 # t0 .. t5
+    for _ in range(4):
+        m.submit(t, [(b, "inout")])                 # t6 .. t9
+    m.load_table([(t, 8, [(10, 1)])])
+    return m
+
+
+def test_critical_path_overtakes_larger_bottom_level():
+    """R38.  0: t0 (bl 6).  10: t1 (bl 5) vs t6 (bl 4) -> t1.  20: t2 (bl 4) ties t6 (bl 4), t2
+    critical -> t2.  30: t3 (bl 3, critical) vs t6 (bl 4, slack 2): critical first -> t3 (by
+    bottom level alone t6 would go at 30 and the chain would end at 100, not 60).  40: t4,
+    50: t5, then the b chain 60-90."""
+    m = _crit_model()
+    assert m.slacks() == [0] * 6 + [2] * 4
+    log = m.simulate(lambda ty, nb, v: 10)
+    assert [(r[0], r[3]) for r in log] == [(0, 0), (1, 10), (2, 20), (3, 30), (4, 40), (5, 50), (6, 60),
+                                           (7, 70), (8, 80), (9, 90)]
 
 
 def test_bottom_level_order_without_queue_cap():

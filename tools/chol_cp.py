@@ -20,7 +20,9 @@ def ids(nt):
 
 def main(path, nt=32, step=-1):
     d = json.load(open(path))
-    log = sorted(d["log"], key=lambda r: r[0])
+    # a combined bench log also holds the matmul's tasks (type 0 = MATMUL): the chain is the
+    # Cholesky's tasks in submission order
+    log = sorted((r for r in d["log"] if r[7] != 0), key=lambda r: r[0])
     n = len(ids(nt))
     steps = [log[i:i + n] for i in range(0, len(log), n)]
     rs = steps[step]
