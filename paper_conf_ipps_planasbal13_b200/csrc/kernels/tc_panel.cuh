@@ -49,11 +49,13 @@ namespace tc {
 // solved (before the cross update), [7 + 2 sb] its cross update done
 #ifdef VS_PANEL_TRACE
 __device__ unsigned long long g_panel_trace[32][32][24];
+__device__ long long g_panel_clk[32][32][24];   // SM clock64 at the same points
 #define PANEL_T(J, i)                                                                  \
     do {                                                                               \
         unsigned long long t_;                                                         \
         asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_));                         \
         g_panel_trace[blockIdx.x & 31][(J) & 31][i] = t_;                              \
+        g_panel_clk[blockIdx.x & 31][(J) & 31][i] = clock64();                         \
     } while (0)
 #else
 #define PANEL_T(J, i)
@@ -622,8 +624,9 @@ inline int tc_potrf(int n, float *A, int lda, int k_base, int *info, cudaStream_
     const unsigned long long id = next_id.fetch_add(1);
     panel_attr<true>();
     count_launch();
-    tc_panel_kernel<true><<<(n + BM - 1) / BM, PTHREADS, PanelCfg::SMEM, s>>>(n, n, A, lda, A, lda, k_base, info, id,
-                                                                             panel_overlap(), 0, 0, ctx);
+    const int grid = (n + BM - 1) / BM;
+    tc_panel_kernel<true><<<grid, PTHREADS, PanelCfg::SMEM, s>>>(n, n, A, lda, A, lda, k_base, info, id,
+                                                                 panel_overlap(), 0, 0, ctx);
     return 0;
 }
 
