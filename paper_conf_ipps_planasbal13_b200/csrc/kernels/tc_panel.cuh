@@ -13,10 +13,10 @@
 //      accumulators (panel parity) so that the MMA of panel J+1 runs while panel J is
 //      being solved.  A operand = the CTA's own solved columns, B operand = the panel's
 //      L rows; the k-blocks that need the columns solved in panel J wait for that panel
-//      only (mbarrier xdone).
+//      only (mbarrier xdone; a per-k-block variant measured slower: 527 vs 490 us).
 //   2. epilogue warps, one row each, per 16-column sub-block sb (compact code: a 16 x 16
 //      step is the only unrolled unit):
-//        x = b - acc[sb]  (b = the tile's current values, prefetched one sub-block ahead);
+//        x = b - acc[sb]  (b = the tile's current values, staged in TMEM by the producers);
 //        TRSM / POTRF below the diagonal: forward substitution against L_JJ staged
 //          (transposed) in shared memory (x_c = t_c / l_cc; t_j -= x_c l_jc);
 //        POTRF diagonal CTA (CTA J holds panel J's diagonal block): per 16-column
@@ -36,6 +36,7 @@
 // representable: integer problems stay exact); sqrt is IEEE.
 #pragma once
 #include <atomic>
+#include <cstdio>
 #include <cstdlib>
 
 #include "tc_gemm.cuh"
@@ -50,12 +51,15 @@ namespace tc {
 #ifdef VS_PANEL_TRACE
 __device__ unsigned long long g_panel_trace[32][32][24];
 __device__ long long g_panel_clk[32][32][24];   // SM clock64 at the same points
+__device__ unsigned long long g_panel_trace_id;  // 0: every launch, else that potrf launch id only
 #define PANEL_T(J, i)                                                                  \
     do {                                                                               \
-        unsigned long long t_;                                                         \
-        asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_));                         \
-        g_panel_trace[blockIdx.x & 31][(J) & 31][i] = t_;                              \
-        g_panel_clk[blockIdx.x & 31][(J) & 31][i] = clock64();                         \
+        if (g_panel_trace_id == 0 || g_panel_trace_id == launch_id) {                  \
+            unsigned long long t_;                                                     \
+            asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t_));                     \
+            g_panel_trace[blockIdx.x & 31][(J) & 31][i] = t_;                          \
+            g_panel_clk[blockIdx.x & 31][(J) & 31][i] = clock64();                     \
+        }                                                                              \
     } while (0)
 #else
 #define PANEL_T(J, i)
@@ -215,7 +219,8 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
     uint64_t *accf = empty + STAGES;   // [2]: accumulator of panel parity b complete
     uint64_t *xdone = accf + 2;        // one phase per panel: its columns solved and stored
     uint64_t *xacc = xdone + 1;        // cross-sub-block update MMAs complete (one phase per use)
-    uint32_t *tmem_slot = (uint32_t *)(xacc + 1);
+    uint64_t *bfull = xacc + 1;        // [2]: b values of panel parity b staged in TMEM (producers)
+    uint32_t *tmem_slot = (uint32_t *)(bfull + 2);
 
     const int m0 = blockIdx.x * BM;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -237,11 +242,13 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
         mbar_init(&accf[1], 1);
         mbar_init(xdone, 4);
         mbar_init(xacc, 1);
+        mbar_init(&bfull[0], 4);
+        mbar_init(&bfull[1], 4);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     }
     if (warp == 0) {
         asm volatile("tcgen05.alloc.cta_group::1.sync.aligned.shared::cta.b32 [%0], %1;" ::"r"(smem_u32(tmem_slot)),
-                     "r"((uint32_t)(2 * P)));
+                     "r"((uint32_t)(4 * P)));
         asm volatile("tcgen05.relinquish_alloc_permit.cta_group::1.sync.aligned;");
     }
     tc_fence_before();
@@ -258,9 +265,39 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
         constexpr int APER = G::APER, BPER = G::BPER;
         const float4 z4 = make_float4(0.f, 0.f, 0.f, 0.f);
         int gkb = 0;
+        // b values of panel J for this thread's row (the tile's current values of the panel's
+        // columns: only this CTA ever writes them, when it solves panel J) -> TMEM columns
+        // [2P + (J & 1) P, +ncols), lane = row: issued while the early k-blocks of panel J are
+        // produced, so the epilogue's x = b - acc reads no global memory on the critical path
+        // (under the GEMM flood the first sub-block's load took 10-15 us)
+        const int brow = m0 + t;
+        const bool browok = brow < rows;
+        auto stage_b = [&](int J) {
+            const int c0 = J * P, ncols = min(P, n - c0);
+            const uint32_t tb = tmem + ((uint32_t)(warp * 32) << 16) + (uint32_t)(2 * P + (J & 1) * P);
+            const float *src = X + (int64_t)(browok ? brow : 0) * ldx + c0;
+            if (browok)   // the row's lines in flight at once; the chunks below then hit L2
+                for (int q0 = 0; q0 < ncols; q0 += 32) asm volatile("prefetch.global.L2 [%0];" ::"l"(src + q0));
+#pragma unroll 1
+            for (int q0 = 0; q0 < ncols; q0 += 16) {   // 16 columns at a time: the k-block
+                float v[16];                            // buffers ra/rb stay live in registers
+#pragma unroll
+                for (int i = 0; i < 4; i++) {
+                    const float4 f = browok ? ld_f4_cg(src + q0 + 4 * i) : z4;
+                    v[4 * i] = f.x; v[4 * i + 1] = f.y; v[4 * i + 2] = f.z; v[4 * i + 3] = f.w;
+                }
+                tmem_st16(tb + q0, v);
+            }
+            tc_fence_before();
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&bfull[J & 1]);
+        };
         for (int J = 0; J < npanels; J++) {
             const int c0 = J * P, nk = c0 / BK;
-            if (nk == 0) continue;
+            if (nk == 0) {
+                stage_b(J);
+                continue;
+            }
             if (POTRF && J != (int)blockIdx.x) {
                 // panel J's L rows (CTA J's) are final once it completed panels < J
                 if (t == 0) wait_flag(&flags[J], tag | (unsigned long long)J);
@@ -268,13 +305,16 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
             }
             if (t == 0) PANEL_T(J, 4);
             // first k-block holding panel J-1's columns (overlap = 0: the whole panel waits)
-            const int kb_new = overlap ? nk - P / BK : 0;
+            const int kb_new = (overlap & 1) ? nk - P / BK : 0;
             constexpr uint32_t idesc = make_idesc(BM, P, false, false);
             const uint32_t dt = tmem + (uint32_t)((J & 1) * P);
             int kbp = 0;   // k-block of this panel being produced
             bool waited = false;
             auto ensure = [&](int kb) {
                 if (kb >= kb_new && !waited) {
+                    // buffer J & 1 was last read by the epilogue in panel J-2: done, since
+                    // these producers passed xdone of panel J-2 in panel J-1
+                    stage_b(J);
                     mbar_wait(xdone, (J - 1) & 1);   // panel J-1 solved and stored
                     waited = true;
                 }
@@ -386,15 +426,22 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 bar_epi();
                 if (e == 0) PANEL_T(J, 1);
             }
-            // b values of sub-block 0 (the tile's current values of the panel columns)
-            float4 bq[4], bn[4];
-#pragma unroll
-            for (int q = 0; q < 4; q++) bq[q] = rowok ? ld_f4_cg(xrow + c0 + 4 * q) : make_float4(0.f, 0.f, 0.f, 0.f);
-            if (nk > 0) {
+            // b values of the panel (staged in TMEM by the producers)
+            const uint32_t tbv = tl + (uint32_t)(2 * P + (J & 1) * P);
+            mbar_wait(&bfull[J & 1], (uint32_t)(J >> 1) & 1u);
+            // POTRF diagonal CTA: one dry pass of the sub-block body (no stores, no MMAs, no
+            // info) while the panel's last MMAs run — the factor code runs only in this CTA's
+            // last panel, and its first execution fetched ~25 KB of instructions from L2:
+            // 2.3 us alone, 15 us under the GEMM flood (PANEL_T)
+            const bool warm = factor && nk > 0 && (overlap & 2);
+            auto acc_ready = [&]() {
                 mbar_wait(&accf[J & 1], (accn >> (J & 1)) & 1u);
                 accn ^= 1u << (J & 1);
                 tc_fence_after();
                 if (e == 0) PANEL_T(J, 2);
+            };
+            if (nk > 0) {
+                if (!warm) acc_ready();
             } else {
                 float z[16];
 #pragma unroll
@@ -403,21 +450,18 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 for (int sb = 0; sb < nsb; sb++) tmem_st16(acc + sb * PSB, z);
             }
 #pragma unroll 1
-            for (int sb = 0; sb < nsb; sb++) {
-                if (sb + 1 < nsb) {
+            for (int sbi = warm ? -1 : 0; sbi < nsb; sbi++) {
+                const bool dry = sbi < 0;
+                const int sb = dry ? 0 : sbi;
+                if (warm && sbi == 0) acc_ready();
+                float x[PSB], bv[PSB];
+                tmem_ld16_issue(acc + sb * PSB, x);
+                tmem_ld16_issue(tbv + sb * PSB, bv);
+                tmem_wait_ld(x);
+                tmem_wait_ld(bv);
 #pragma unroll
-                    for (int q = 0; q < 4; q++)
-                        bn[q] = rowok ? ld_f4_cg(xrow + c0 + (sb + 1) * PSB + 4 * q) : make_float4(0.f, 0.f, 0.f, 0.f);
-                }
-                float x[PSB];
-                tmem_ld16(acc + sb * PSB, x);
-#pragma unroll
-                for (int q = 0; q < 4; q++) {
-                    x[4 * q + 0] = bq[q].x - x[4 * q + 0];
-                    x[4 * q + 1] = bq[q].y - x[4 * q + 1];
-                    x[4 * q + 2] = bq[q].z - x[4 * q + 2];
-                    x[4 * q + 3] = bq[q].w - x[4 * q + 3];
-                }
+                for (int i = 0; i < PSB; i++) x[i] = bv[i] - x[i];
+                if (e == 0 && sbi == 0) PANEL_T(J, 22);
                 if (factor) {
                     // the 16 x 16 diagonal sub-block is factored by the warp holding its rows,
                     // with shuffles (no block barrier per column); its L is published in Lt/Lr,
@@ -435,7 +479,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                             // selects, not branches: under `r == c` the compiler would rewrite
                             // x[c] as x[r], a dynamic index that sends x[] to local memory
                             const bool piv_row = drow && r == c;
-                            if (piv_row && !(piv > 0.f) && info) atomicCAS(info, 0, k_base + c0 + d0 + c + 1);
+                            if (piv_row && !(piv > 0.f) && info && !dry) atomicCAS(info, 0, k_base + c0 + d0 + c + 1);
                             const float xd = div_nr(x[c], l, rcp_approx(l));
                             x[c] = piv_row ? l : ((drow && r > c) ? xd : x[c]);
                             dg = piv_row ? l : dg;
@@ -451,7 +495,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                                 }
                             }
                         }
-                        if (drow) {
+                        if (drow && !dry) {
 #pragma unroll
                             for (int c = 0; c < PSB; c++) Lt[(d0 + c) * LD + e] = x[c];
                             Lr[e] = rcp_approx(dg);
@@ -467,8 +511,9 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                             for (int j = c + 1; j < PSB; j++) x[j] = fmaf(-x[c], Lt[cc * LD + d0 + j], x[j]);
                         }
                         // publish this row's L_JJ values (transposed) for the cross updates
+                        if (!dry)
 #pragma unroll
-                        for (int c = 0; c < PSB; c++) Lt[(d0 + c) * LD + e] = x[c];
+                            for (int c = 0; c < PSB; c++) Lt[(d0 + c) * LD + e] = x[c];
                     }
                     bar_epi();
                 } else {
@@ -480,6 +525,8 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                         for (int j = c + 1; j < PSB; j++) x[j] = fmaf(-x[c], Lt[cc * LD + sb * PSB + j], x[j]);
                     }
                 }
+                if (e == 0 && sbi == 0) PANEL_T(J, 23);
+                if (dry) continue;
                 // store the solved row segment (diagonal block: lower part only)
                 if (rowok) {
                     float *dst = xrow + c0 + sb * PSB;
@@ -541,8 +588,6 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     tc_fence_after();
                 }
                 if (e == 0) PANEL_T(J, 7 + 2 * sb);
-#pragma unroll
-                for (int q = 0; q < 4; q++) bq[q] = bn[q];
             }
             if (e == 0) PANEL_T(J, 3);
             // panel J of these rows: visible at L2 (own producers, other CTAs), TMEM reads done
@@ -561,18 +606,20 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
     __syncthreads();
     tc_fence_after();
     if (warp == 0) {
-        asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)(2 * P)));
+        asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"((uint32_t)(4 * P)));
     }
     ctx_end(ctx);
 }
 
-// MMA of panel J+1 overlapped with the solve of panel J (default); VS_PANEL_OVERLAP=0
-// serialises them (measurement switch)
+// kernel option bits (measurement switches): bit 0 — MMA of panel J+1 overlapped with the
+// solve of panel J (default; VS_PANEL_OVERLAP=0 serialises them); bit 1 — the diagonal CTA's
+// dry pass of the factor code (default; VS_PANEL_WARM=0 disables)
 inline int panel_overlap()
 {
     static const int v = [] {
         const char *e = getenv("VS_PANEL_OVERLAP");
-        return e ? atoi(e) : 1;
+        const char *w = getenv("VS_PANEL_WARM");
+        return (e ? (atoi(e) ? 1 : 0) : 1) | ((w ? (atoi(w) ? 1 : 0) : 1) << 1);
     }();
     return v;
 }
@@ -622,6 +669,29 @@ inline int tc_potrf(int n, float *A, int lda, int k_base, int *info, cudaStream_
     if (n % 64 || (n + BM - 1) / BM > kFlagCtas) return -1;
     static std::atomic<unsigned long long> next_id{1};
     const unsigned long long id = next_id.fetch_add(1);
+#ifdef VS_PANEL_TRACE
+    // one potrf of a whole run (VS_TRACE_POTRF = its launch id), dumped at exit to VS_TRACE_FILE
+    static const unsigned long long want = [] {
+        const char *e = getenv("VS_TRACE_POTRF");
+        const unsigned long long w = e ? strtoull(e, nullptr, 10) : 0;
+        cudaMemcpyToSymbol(g_panel_trace_id, &w, sizeof w);
+        if (w) atexit([] {
+            static unsigned long long tr[32][32][24];
+            static long long ck[32][32][24];
+            cudaDeviceSynchronize();
+            cudaMemcpyFromSymbol(tr, g_panel_trace, sizeof tr);
+            cudaMemcpyFromSymbol(ck, g_panel_clk, sizeof ck);
+            const char *f = getenv("VS_TRACE_FILE");
+            if (FILE *fp = fopen(f ? f : "panel_trace.bin", "wb")) {
+                fwrite(tr, sizeof tr, 1, fp);
+                fwrite(ck, sizeof ck, 1, fp);
+                fclose(fp);
+            }
+        });
+        return w;
+    }();
+    (void)want;
+#endif
     panel_attr<true>();
     count_launch();
     const int grid = (n + BM - 1) / BM;
