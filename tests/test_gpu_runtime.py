@@ -128,6 +128,21 @@ def test_equally_critical_chains_run_concurrently(gpu):
     rt.close()
 
 
+def test_lone_matmul_keeps_grouped_launches(gpu):
+    # every task of a lone matmul has slack 0 (R33/R38); in the bench configuration its
+    # tc_3xf16 tasks must still share grouped launches (a flush of every critical task on its
+    # own once ungrouped the whole matmul: 317 -> 123 TFLOP/s in the bench)
+    import bench
+    rt = vs.Runtime(bench.bench_config(vs, lam=1))
+    s0 = rt.vs_stats()
+    A, B, C0, C = _matmul(rt, 2048, 256, mask=1 << vs.VS_V_TC_3XF16)
+    s1 = rt.vs_stats()
+    launches = s1.group_launches - s0.group_launches
+    assert launches > 0 and 512 / launches >= 2.0, launches
+    assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-5
+    rt.close()
+
+
 def test_matmul_f64_family(gpu):
     rt = vs.Runtime(lam=1)
     mask = (1 << vs.VS_V_DFMA_F64) | (1 << vs.VS_V_DMMA_F64)
