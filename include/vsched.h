@@ -188,13 +188,23 @@ typedef struct {
     void *(*dev_alloc)(int device, size_t bytes, void *user);
     void (*dev_free)(int device, void *ptr, void *user);
     void *alloc_user;
+    int stage;         /* n > 0 (default 32): transfer-ordered drive (reading R39; L515-532) — when a
+                          fresh batch in ready mode with priority 2 on one GPU of one process reads
+                          data homed in host memory, a list schedule of the batch fixes the order
+                          in which those inputs cross the host link (critical path first, then
+                          fewest unplanned input bytes, then the datum closest to its final
+                          version, then weighted bottom level); the runtime copies them in that
+                          order with at most n copies in flight, uses the planned position as the
+                          ready order, and decides a task only once its inputs have arrived.
+                          0: inputs move on demand when their reader is issued.  VS_STAGE=n
+                          overrides */
 } vs_config;
 
 /* Fill *cfg with defaults: GPU, 1 gpu, base 0, 4 slots, lambda 3, versioning, hold,
  * run-ahead, live timing, flush.  Environment overrides applied by vs_create (L277-288):
  * VS_LAMBDA, VS_SLOTS, VS_POLICY(=versioning|fixed:<v>), VS_LEARNING(=hold|rr),
  * VS_MODE(=runahead|ready), VS_LOOKAHEAD(=n), VS_PRIORITY(=0|1|2), VS_QDEPTH(=d), VS_GROUP_HOLD(=0|1),
- * VS_GROUP(=tasks per grouped launch), VS_GROUP_US.  Runtime options outside vs_config:
+ * VS_GROUP(=tasks per grouped launch), VS_GROUP_US, VS_STAGE(=n).  Runtime options outside vs_config:
  * VS_TRACKER(=events|memops) dependence tracker on one GPU, VS_GROUP_DIST(=0|1, default 1)
  * grouped launches in a multi-rank job, VS_PREFETCH(=n, default 0) input-prefetch window on one
  * GPU, VS_TCF_PAIR(=0|1, default 1) CTA-pair variant of the tc_3xf16 GEMM. */
@@ -304,6 +314,8 @@ typedef struct {
     int64_t device_released;  /* tasks made ready by the device dependence tracker (a3) */
     int64_t host_ns_group_launch; /* host time inside grouped kernel launches */
     int64_t group_launches;   /* grouped kernel launches issued */
+    int64_t gated_tasks;      /* ready tasks that waited for their host inputs to arrive before
+                                 being decided (transfer-ordered drive, vs_config.stage) */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 
@@ -369,6 +381,12 @@ int vs_app_matmul(vs_rt rt, vs_type_id matmul_type, int m, int l, int n,
 /* Right-looking lower tiled Cholesky (R5): A[i*nt+j] for i >= j, types[VS_T_*]. */
 int vs_app_cholesky(vs_rt rt, const vs_type_id types[VS_NUM_BUILTIN_TYPES], int nt,
                     const vs_data_id *A);
+/* Transfer plan of the submitted batch before it starts (vs_config.stage, reading R39): the ids
+ * of the host-homed data it reads, in the order a transfer-ordered drive copies them to the
+ * GPU.  Writes min(cap, total) ids to out (caller-owned; may be NULL when cap = 0) and the
+ * total to *n (0 when no task of the batch reads host-only data).  Starts nothing; any
+ * executor.  VS_E_STATE once the batch has started (a wait has driven it). */
+int vs_transfer_plan(vs_rt rt, vs_data_id *out, int64_t cap, int64_t *n);
 
 /* ----------------------------------------------------- direct tile kernels */
 /* Enqueue one built-in tile task version on `stream` on the current device, outside

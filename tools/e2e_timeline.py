@@ -30,8 +30,17 @@ def main(only="both"):
     log = rt.vs_decision_log()
     d0 = min(r[4] for r in log)
     ends = max(r[5] for r in log)
-    print("wall %.1f ms; device span of the tasks %.1f ms; H2D %.2f GB, D2H %.2f GB" % (
-        wall, (ends - d0) / 1e6, (s1.input_tx_bytes - s0.input_tx_bytes) / 1e9, (s1.output_tx_bytes - s0.output_tx_bytes) / 1e9))
+    print("wall %.1f ms; device span of the tasks %.1f ms; H2D %.2f GB, D2H %.2f GB; %d tasks gated on inputs" % (
+        wall, (ends - d0) / 1e6, (s1.input_tx_bytes - s0.input_tx_bytes) / 1e9, (s1.output_tx_bytes - s0.output_tx_bytes) / 1e9,
+        s1.gated_tasks - s0.gated_tasks))
+    for _ in range(2):
+        wl.reset()
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        wl.submit()
+        rt.vs_wait_all()
+        torch.cuda.synchronize()
+        print("  again: wall %.1f ms" % ((time.perf_counter() - t0) * 1e3))
     names = {0: "mm"}
     bins = {}
     for r in log:
@@ -41,6 +50,26 @@ def main(only="both"):
         bins[k][b] += 1
     for k, h in bins.items():
         print(k, "tasks started per 5 ms:", " ".join("%d" % h.get(i, 0) for i in range(max(h) + 1)))
+    ct = os.environ.get("VS_COPY_TRACE")
+    if ct and os.path.exists(ct):   # copy completions of the timed step (first block after warm-up)
+        blocks, cur = [], []
+        for line in open(ct):
+            if line.startswith("#"):
+                blocks.append(cur)
+                cur = []
+            else:
+                k, t, b = line.split()
+                cur.append((int(k), float(t), int(b)))
+        if len(blocks) >= 3:
+            blk = blocks[2]
+            for kind, name in ((0, "H2D"), (1, "D2H")):
+                h = {}
+                for k, t, b in blk:
+                    if k == kind:
+                        h[int(t / 5000)] = h.get(int(t / 5000), 0) + b
+                if h:
+                    print(name, "GB/s per 5 ms:", " ".join("%.0f" % (h.get(i, 0) / 5e-3 / 1e9) for i in range(max(h) + 1)),
+                          "| last %.1f ms" % (max(t for k, t, b in blk if k == kind) / 1e3))
     busy = sum(r[5] - r[4] for r in log) / 1e6
     print("summed task time %.1f ms (concurrent tasks overlap)" % busy)
     rt.close()
