@@ -389,3 +389,19 @@ int launch_builtin(int type, int version, int b, void *const *p, int *info, cuda
 }
 
 }  // namespace vsk
+
+#ifdef VS_TCF_TRACE
+// measurement builds only: read (and reset) the tc_3xf16 GEMM's per-CTA phase records
+extern "C" __attribute__((visibility("default"))) int vs_debug_tcf_trace(unsigned long long *out, int cap)
+{
+    unsigned int n = 0;
+    cudaDeviceSynchronize();
+    cudaMemcpyFromSymbol(&n, vsk::tcf::g_tcf_n, sizeof n);
+    if (n > (unsigned)vsk::tcf::kTcfTraceCap) n = vsk::tcf::kTcfTraceCap;
+    if (n > (unsigned)cap) n = (unsigned)cap;
+    if (n) cudaMemcpyFromSymbol(out, vsk::tcf::g_tcf_rec, (size_t)n * 12 * sizeof(unsigned long long));
+    unsigned int z = 0;
+    cudaMemcpyToSymbol(vsk::tcf::g_tcf_n, &z, sizeof z);
+    return (int)n;
+}
+#endif

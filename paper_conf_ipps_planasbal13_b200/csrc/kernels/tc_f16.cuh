@@ -67,18 +67,36 @@ using tc::tc_fence_before;
 using tc::tmem_ld32;
 using tc::tmem_st32;
 
-// Optional per-CTA phase timeline (tools/probe_tcf.cu builds with -DVS_TCF_TRACE).
+// Optional per-CTA phase timeline (measurement builds with -DVS_TCF_TRACE, tools/tcf_trace.py):
+// every CTA of every launch appends {%globaltimer at: 0 start, 1 TMEM allocated, 2 first stage
+// full, 3 half of the k-blocks, 4 last MMAs issued, 5 epilogue ready, 6 accumulator full,
+// 8 epilogue done, 10 CTA end; 9 = total ns the MMA warp waited for full stages; 11 = SM id}
+// to a device ring read back with vs_debug_tcf_trace.
 #ifdef VS_TCF_TRACE
-__device__ unsigned long long g_tcf_trace[1024][12];
-#define TCF_T(i) g_tcf_trace[blockIdx.y * gridDim.x + blockIdx.x][i] = tc_now()
-#define TCF_ADD(i, v) g_tcf_trace[blockIdx.y * gridDim.x + blockIdx.x][i] += (v)
+constexpr int kTcfTraceCap = 1 << 17;
+__device__ unsigned long long g_tcf_rec[kTcfTraceCap][12];
+__device__ unsigned int g_tcf_n;
+#define TCF_DECL __shared__ unsigned long long s_tcf[12]
+#define TCF_T(i) s_tcf[i] = tc_now()
+#define TCF_ADD(i, v) s_tcf[i] += (v)
 __device__ __forceinline__ unsigned long long tc_now()
 {
     unsigned long long t;
     asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
     return t;
 }
+__device__ __forceinline__ void tcf_trace_flush(unsigned long long (&s)[12])
+{
+    unsigned int smid;
+    asm volatile("mov.u32 %0, %smid;" : "=r"(smid));
+    s[10] = tc_now();
+    s[11] = smid;
+    const unsigned int i = atomicAdd(&g_tcf_n, 1u);
+    if (i < kTcfTraceCap)
+        for (int k = 0; k < 12; k++) g_tcf_rec[i][k] = s[k];
+}
 #else
+#define TCF_DECL
 #define TCF_T(i)
 #define TCF_ADD(i, v)
 #endif
@@ -339,6 +357,7 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
 {
     extern __shared__ uint8_t smem_raw[];
     uint8_t *smem = smem_raw + ((1024u - (smem_u32(smem_raw) & 1023u)) & 1023u);
+    TCF_DECL;
     uint64_t *full = (uint64_t *)(smem + STAGES * STAGE);
     uint64_t *empty = full + STAGES;
     uint64_t *acc_full = empty + STAGES;
@@ -391,6 +410,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
 
     if (threadIdx.x == 0) {
         TCF_T(0);
+#ifdef VS_TCF_TRACE
+        s_tcf[9] = 0;
+#endif
         for (int s = 0; s < STAGES; s++) {
             mbar_init(&full[s], 1);
             mbar_init(&empty[s], PAIR ? 2 : 1);
@@ -551,6 +573,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         asm volatile("tcgen05.dealloc.cta_group::1.sync.aligned.b32 %0, %1;" ::"r"(tmem), "r"(512u));
     }
     if (PAIR) cluster_sync_all();   // no CTA leaves while its peer may still address its smem
+#ifdef VS_TCF_TRACE
+    if (threadIdx.x == 0) tcf_trace_flush(s_tcf);
+#endif
     ctx_end(ctx);
 }
 
