@@ -211,8 +211,14 @@ class Workload:
         # the restores run on the GPU while the host builds the step's task graph (vs_submit
         # only records tasks and dependences; nothing is issued before vs_wait_all)
         self.reset(sync=False)
+        if not self.host and barrier is None and not os.environ.get("VS_BENCH_SYNC"):
+            # one process: the runtime's streams wait for the restore on the device
+            # (vs_depend_on_event), so the drive's host-side setup overlaps it
+            self._ev = self.torch.cuda.Event()
+            self._ev.record()
+            self.rt.vs_depend_on_event(self._ev)
         self.submit()
-        if not self.host:
+        if not self.host and (barrier is not None or os.environ.get("VS_BENCH_SYNC")):
             self.torch.cuda.current_stream().synchronize()
         if barrier:
             barrier()      # owners' resets done before any rank reads their tiles

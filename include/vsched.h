@@ -316,6 +316,9 @@ typedef struct {
     int64_t group_launches;   /* grouped kernel launches issued */
     int64_t gated_tasks;      /* ready tasks that waited for their host inputs to arrive before
                                  being decided (transfer-ordered drive, vs_config.stage) */
+    int64_t host_ns_drive_setup; /* host time from entering a wait's drive to its first
+                                 decisions issued (dependence tracker upload, bottom levels,
+                                 transfer plan) */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 
@@ -381,6 +384,13 @@ int vs_app_matmul(vs_rt rt, vs_type_id matmul_type, int m, int l, int n,
 /* Right-looking lower tiled Cholesky (R5): A[i*nt+j] for i >= j, types[VS_T_*]. */
 int vs_app_cholesky(vs_rt rt, const vs_type_id types[VS_NUM_BUILTIN_TYPES], int nt,
                     const vs_data_id *A);
+/* Order the next drive (the device work of the next vs_wait_*) after a CUDA event the caller
+ * recorded on its own stream (cudaEvent_t passed as void*; the caller keeps it alive until
+ * that wait returns), e.g. the kernels that produced the batch's device-homed inputs: every
+ * stream of the runtime waits for it on the device, so the runtime's host-side setup of the
+ * drive (dependence tracker upload, bottom levels, transfer plan) overlaps the caller's work
+ * instead of following a host synchronisation.  Consumed by that drive.  No-op in SIM. */
+int vs_depend_on_event(vs_rt rt, void *cuda_event);
 /* Transfer plan of the submitted batch before it starts (vs_config.stage, reading R39): the ids
  * of the host-homed data it reads, in the order a transfer-ordered drive copies them to the
  * GPU.  Writes min(cap, total) ids to out (caller-owned; may be NULL when cap = 0) and the

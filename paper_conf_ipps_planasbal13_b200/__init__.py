@@ -56,7 +56,7 @@ class vs_stats_t(Structure):
         "tasks_submitted", "tasks_completed", "decisions", "input_tx_bytes", "output_tx_bytes", "device_tx_bytes",
         "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns",
         "kernel_launches", "tracker", "forms_built", "host_ns_poll", "host_ns_launch", "host_ns_deps", "host_loops", "host_ns_vevent", "host_ns_flush",
-        "host_idle_loops", "device_released", "host_ns_group_launch", "group_launches", "gated_tasks")]
+        "host_idle_loops", "device_released", "host_ns_group_launch", "group_launches", "gated_tasks", "host_ns_drive_setup")]
 
 
 class vs_group_stat_t(Structure):
@@ -120,6 +120,7 @@ def lib():
                                   POINTER(c_int64)]),
         "vs_app_cholesky": (c_int, [rt, POINTER(c_int32), c_int, POINTER(c_int64)]),
         "vs_transfer_plan": (c_int, [rt, POINTER(c_int64), c_int64, POINTER(c_int64)]),
+        "vs_depend_on_event": (c_int, [rt, c_void_p]),
         "vs_tile_run": (c_int, [c_int, c_int, c_int, POINTER(c_void_p), c_void_p, c_void_p]),
         "vs_gen_uniform": (c_int, [c_uint64, c_int64, c_int64, c_int, c_int, c_void_p, c_void_p]),
         "vs_gen_spd": (c_int, [c_uint64, c_int64, c_int, c_int, c_void_p, c_void_p]),
@@ -151,7 +152,7 @@ EXPORTED = ["vs_config_default", "vs_create", "vs_destroy", "vs_last_error", "vs
             "vs_register_builtins", "vs_data_register", "vs_submit", "vs_wait_all", "vs_wait_all_noflush",
             "vs_wait_on", "vs_stats", "vs_group_count", "vs_group_stat", "vs_type_name", "vs_version_name",
             "vs_decision_log", "vs_decision_log_hash", "vs_decision_log_clear", "vs_table_dump", "vs_table_load",
-            "vs_replay_set", "vs_app_matmul", "vs_app_cholesky", "vs_transfer_plan", "vs_tile_run", "vs_gen_uniform", "vs_gen_spd",
+            "vs_replay_set", "vs_app_matmul", "vs_app_cholesky", "vs_transfer_plan", "vs_depend_on_event", "vs_tile_run", "vs_gen_uniform", "vs_gen_spd",
             "vs_build_info", "vs_gen_tile", "vs_dist_init", "vs_data_set_owner", "vs_ipc_export", "vs_ipc_open",
             "vs_ipc_close", "vs_data_invalidate", "vs_data_invalidate_n", "vs_operand_form", "vs_form_bytes", "vs_form_make",
             "vs_tile_run_prepared", "vs_decision_issue_ns", "vs_gpu_ordinal"]
@@ -381,6 +382,11 @@ class Runtime:
         buf = (c_int64 * max(1, n.value))()
         lib().vs_decision_issue_ns(self.h, buf, n.value, ctypes.byref(n))
         return list(buf[:n.value])
+
+    def vs_depend_on_event(self, event):
+        """The next drive's device work waits for `event` (a torch.cuda.Event or a raw cudaEvent_t)."""
+        h = getattr(event, "cuda_event", event)
+        return self._ck(lib().vs_depend_on_event(self.h, c_void_p(int(h))), "vs_depend_on_event")
 
     def vs_transfer_plan(self):
         """Data ids of the batch's host-homed inputs in transfer order (vs_transfer_plan)."""

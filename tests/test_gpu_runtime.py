@@ -111,6 +111,44 @@ def test_host_data_bench_config_eager_writeback(gpu):
     rt.close()
 
 
+@pytest.mark.parametrize("stage", [32, 1, 0])
+def test_staged_host_batch_matmul_and_cholesky(gpu, stage):
+    # transfer-ordered drive (R39): a matmul and a Cholesky with host-homed tiles in one batch;
+    # the inputs cross the link in the planned order (window of `stage` copies, 1 = one at a
+    # time), tasks wait for their inputs in the ready queue, results as without staging
+    import torch
+
+    import bench
+    rt = vs.Runtime(bench.bench_config(vs, lam=1, slots_per_gpu=4, stage=stage))
+    mask = (1 << vs.VS_V_TC_3XTF32) | (1 << vs.VS_V_TC_3XF16)
+    types = rt.vs_register_builtins(vs.VS_F32, mask)
+    Nm, bm, Nc, bc = 1024, 256, 2048, 256
+    A, B = vsgen.uniform(81, Nm, Nm), vsgen.uniform(82, Nm, Nm)
+    C0 = vsgen.uniform(83, Nm, Nm)
+    tA, tB, tC = (torch.from_numpy(vsgen.to_tiles(x, bm)).pin_memory() for x in (A, B, C0))
+    ia, ib, ic = (_register_tiles(rt, t, -1) for t in (tA, tB, tC))
+    S = vsgen.spd(84, Nc)
+    nt = Nc // bc
+    T = torch.from_numpy(vsgen.to_tiles(S, bc)).pin_memory()
+    ids = {i * nt + j: rt.vs_data_register(T[i, j].data_ptr(), -1, bc * bc * 4) for i in range(nt) for j in range(i + 1)}
+    rt.vs_app_matmul(types[vs.VS_T_MATMUL], 4, 4, 4, ia, ib, ic)
+    rt.vs_app_cholesky(types, nt, ids)
+    plan = rt.vs_transfer_plan()
+    assert len(plan) == 48 + len(ids) and len(set(plan)) == len(plan)
+    assert set(plan[:len(ids)]) == set(ids.values())       # the longer chain's inputs first
+    rt.vs_wait_all()
+    C = vsgen.from_tiles(tC.numpy())
+    assert oracle.relF(C, oracle.matmul(A, B, C0)) <= 1e-5
+    L = np.tril(vsgen.from_tiles(T.numpy()))
+    Lref, info = oracle.cholesky(S)
+    assert info == 0 and oracle.relF(L, Lref) <= 1e-5
+    st = rt.vs_stats()
+    assert st.input_tx_bytes == len(plan) * bm * bm * 4
+    assert st.output_tx_bytes == (16 + len(ids)) * bm * bm * 4
+    assert (st.gated_tasks > 0) == (stage > 0)
+    rt.close()
+
+
 def test_equally_critical_chains_run_concurrently(gpu):
     # R33: in the bench configuration (bottom-level priority, critical-path streams) a lone
     # matmul has 16 equally critical k-chains; they must run side by side, not queue on the

@@ -43,8 +43,10 @@ def main():
         rt.vs_wait_all()
         t5 = time.perf_counter()
         s1 = rt.vs_stats()
-        print("restore-enqueue %.2f ms  invalidate %.2f  submit %.2f  sync %.2f  wait_all %.2f  (decide+issue+poll+flush %.1f ms)"
+        print("restore-enqueue %.2f ms  invalidate %.2f  submit %.2f  sync %.2f  wait_all %.2f  (drive setup %.2f ms;"
+              " decide+issue+poll+flush %.1f ms)"
               % ((t1 - t0) * 1e3, (t2 - t1) * 1e3, (t3 - t2) * 1e3, (t4 - t3) * 1e3, (t5 - t4) * 1e3,
+                 (s1.host_ns_drive_setup - s0.host_ns_drive_setup) / 1e6,
                  (s1.host_ns_poll - s0.host_ns_poll + s1.host_ns_flush - s0.host_ns_flush) / 1e6))
     rt.close()
 
