@@ -220,7 +220,8 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
     uint64_t *xdone = accf + 2;        // one phase per panel: its columns solved and stored
     uint64_t *xacc = xdone + 1;        // cross-sub-block update MMAs complete (one phase per use)
     uint64_t *bfull = xacc + 1;        // [2]: b values of panel parity b staged in TMEM (producers)
-    uint32_t *tmem_slot = (uint32_t *)(bfull + 2);
+    uint64_t *pstart = bfull + 2;      // POTRF feed: the producers issued the factor panel's first MMAs
+    uint32_t *tmem_slot = (uint32_t *)(pstart + 1);
 
     const int m0 = blockIdx.x * BM;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -244,6 +245,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
         mbar_init(xacc, 1);
         mbar_init(&bfull[0], 4);
         mbar_init(&bfull[1], 4);
+        mbar_init(pstart, 1);
         asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     }
     if (warp == 0) {
@@ -258,6 +260,16 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
     // panels this CTA takes part in: POTRF stops at the panel holding its rows' diagonal
     int npanels = (n + P - 1) / P;
     if (POTRF) npanels = min(npanels, (int)blockIdx.x + 1);
+    // POTRF feed (option bit 2): the factor panel's update by the previous panel,
+    // A_cc -= L_c,c-1 L_c,c-1^T, uses this CTA's own rows for both operands, so the epilogue
+    // issues it sub-block by sub-block while it solves panel c-1 (operands already staged for
+    // the cross-sub-block update) instead of the producers reloading the solved columns from
+    // global memory after the whole panel is stored: the accumulator of the factor panel is
+    // ready as soon as the solve ends (critical chain of the factorisation)
+    const int fpanel = (int)blockIdx.x;
+    const bool feed = POTRF && (overlap & 4) && (overlap & 1) && fpanel >= 1 && fpanel < npanels + 0 &&
+                      fpanel * P < n;
+    const bool feed_pk = feed && fpanel * P / BK - P / BK > 0;   // the producers issue MMAs of the factor panel
 
     if (warp < 4) {
         // =================================================== producers
@@ -293,9 +305,12 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
             if (lane == 0) mbar_arrive(&bfull[J & 1]);
         };
         for (int J = 0; J < npanels; J++) {
-            const int c0 = J * P, nk = c0 / BK;
+            const int c0 = J * P;
+            // feed: the factor panel's k-blocks of panel J-1 are issued by the epilogue instead
+            const int nk = (feed && J == fpanel) ? c0 / BK - P / BK : c0 / BK;
             if (nk == 0) {
                 stage_b(J);
+                if (feed && J == fpanel && threadIdx.x == 0) mma_commit(&accf[J & 1]);   // nothing of the producers' to wait for
                 continue;
             }
             if (POTRF && J != (int)blockIdx.x) {
@@ -304,8 +319,9 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 asm volatile("bar.sync 1, 128;" ::: "memory");
             }
             if (t == 0) PANEL_T(J, 4);
-            // first k-block holding panel J-1's columns (overlap = 0: the whole panel waits)
-            const int kb_new = (overlap & 1) ? nk - P / BK : 0;
+            // first k-block holding panel J-1's columns (overlap = 0: the whole panel waits); with
+            // the feed the factor panel has none of them
+            const int kb_new = (feed && J == fpanel) ? nk : (overlap & 1) ? nk - P / BK : 0;
             constexpr uint32_t idesc = make_idesc(BM, P, false, false);
             const uint32_t dt = tmem + (uint32_t)((J & 1) * P);
             int kbp = 0;   // k-block of this panel being produced
@@ -372,6 +388,10 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                         }
                         mma_commit(&empty[s]);
                         if (kbp == nk - 1) mma_commit(&accf[J & 1]);
+                        if (feed && J == fpanel && kbp == 0) {   // the accumulator is initialised
+                            tc_fence_before();
+                            mbar_arrive(pstart);
+                        }
                     }
                     __syncwarp();
                 }
@@ -389,6 +409,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     if (kb + 3 < nk) load(ra1, rb1, kb + 3);
                 }
             }
+            if (feed && J == fpanel) stage_b(J);   // (no k-block reached kb_new)
             if (t == 0) PANEL_T(J, 5);
         }
     } else {
@@ -546,7 +567,8 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 // one epilogue thread into the panel's TMEM accumulator, operands staged in the
                 // XS area (SW64 K-major: A = the 128 rows' 16 solved values, B = rows of L_JJ)
                 if (e == 0) PANEL_T(J, 6 + 2 * sb);
-                if (sb + 1 < nsb) {
+                const bool feed_j = feed && J + 1 == fpanel;
+                if (sb + 1 < nsb || feed_j) {
                     const int nb = (nsb - sb - 1) * PSB;   // later columns (a multiple of 16)
                     {   // A: this row's values, split big / small
                         const uint32_t ra = (uint32_t)e * 64u;
@@ -556,7 +578,7 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                             store_split(xs_ab, xs_as, off, make_float4(x[4 * q], x[4 * q + 1], x[4 * q + 2], x[4 * q + 3]));
                         }
                     }
-                    if (e < nb) {   // B: row (sb+1)*16 + e of L_JJ, columns sb*16 .. +15 (from Lt)
+                    if (e < nb && sb + 1 < nsb) {   // B: row (sb+1)*16 + e of L_JJ, columns sb*16 .. +15 (from Lt)
                         const float *lc = Lt + (sb * PSB) * LD + (sb + 1) * PSB + e;
                         const uint32_t rb = (uint32_t)e * 64u;
 #pragma unroll
@@ -571,15 +593,36 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     bar_epi();
                     if (e == 0) {
                         tc_fence_after();
-                        const uint32_t idesc = make_idesc(BM, nb, false, false);
-                        const uint32_t d = tmem + (uint32_t)((J & 1) * P + (sb + 1) * PSB);
                         const uint32_t ab = smem_u32(xs_ab), as = smem_u32(xs_as), bb = smem_u32(xs_bb), bs = smem_u32(xs_bs);
+                        if (sb + 1 < nsb) {
+                            const uint32_t idesc = make_idesc(BM, nb, false, false);
+                            const uint32_t d = tmem + (uint32_t)((J & 1) * P + (sb + 1) * PSB);
 #pragma unroll
-                        for (int kk = 0; kk < PSB / 8; kk++) {
-                            const uint32_t o = kk * 32;
-                            mma_tf32(d, desc_sw64(ab + o), desc_sw64(bb + o), idesc, 1u);
-                            mma_tf32(d, desc_sw64(ab + o), desc_sw64(bs + o), idesc, 1u);
-                            mma_tf32(d, desc_sw64(as + o), desc_sw64(bb + o), idesc, 1u);
+                            for (int kk = 0; kk < PSB / 8; kk++) {
+                                const uint32_t o = kk * 32;
+                                mma_tf32(d, desc_sw64(ab + o), desc_sw64(bb + o), idesc, 1u);
+                                mma_tf32(d, desc_sw64(ab + o), desc_sw64(bs + o), idesc, 1u);
+                                mma_tf32(d, desc_sw64(as + o), desc_sw64(bb + o), idesc, 1u);
+                            }
+                        }
+                        if (feed_j) {
+                            // acc[factor panel] += x_sb x_sb^T: these rows are the factor panel's
+                            // rows and columns (A = B = the staged x block), after the producers'
+                            // first (initialising) MMA of that panel
+                            if (sb == 0 && feed_pk) {
+                                mbar_wait(pstart, 0);
+                                tc_fence_after();
+                            }
+                            const uint32_t idesc = make_idesc(BM, P, false, false);
+                            const uint32_t d = tmem + (uint32_t)(((J + 1) & 1) * P);
+#pragma unroll
+                            for (int kk = 0; kk < PSB / 8; kk++) {
+                                const uint32_t o = kk * 32;
+                                const uint32_t init = (!feed_pk && sb == 0 && kk == 0) ? 0u : 1u;
+                                mma_tf32(d, desc_sw64(ab + o), desc_sw64(ab + o), idesc, init);
+                                mma_tf32(d, desc_sw64(ab + o), desc_sw64(as + o), idesc, 1u);
+                                mma_tf32(d, desc_sw64(as + o), desc_sw64(ab + o), idesc, 1u);
+                            }
                         }
                         mma_commit(xacc);
                     }
@@ -613,13 +656,15 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
 
 // kernel option bits (measurement switches): bit 0 — MMA of panel J+1 overlapped with the
 // solve of panel J (default; VS_PANEL_OVERLAP=0 serialises them); bit 1 — the diagonal CTA's
-// dry pass of the factor code (default; VS_PANEL_WARM=0 disables)
+// dry pass of the factor code (default; VS_PANEL_WARM=0 disables); bit 2 — POTRF feed of the
+// factor panel's accumulator by the previous panel's solve (default; VS_PANEL_FEED=0 disables)
 inline int panel_overlap()
 {
     static const int v = [] {
         const char *e = getenv("VS_PANEL_OVERLAP");
         const char *w = getenv("VS_PANEL_WARM");
-        return (e ? (atoi(e) ? 1 : 0) : 1) | ((w ? (atoi(w) ? 1 : 0) : 1) << 1);
+        const char *f = getenv("VS_PANEL_FEED");
+        return (e ? (atoi(e) ? 1 : 0) : 1) | ((w ? (atoi(w) ? 1 : 0) : 1) << 1) | ((f ? (atoi(f) ? 1 : 0) : 1) << 2);
     }();
     return v;
 }

@@ -23,6 +23,7 @@ def main(only="both"):
     torch.cuda.synchronize()
     t0 = time.perf_counter()
     wl.submit()
+    sub = (time.perf_counter() - t0) * 1e3
     rt.vs_wait_all()
     torch.cuda.synchronize()
     wall = (time.perf_counter() - t0) * 1e3
@@ -30,9 +31,11 @@ def main(only="both"):
     log = rt.vs_decision_log()
     d0 = min(r[4] for r in log)
     ends = max(r[5] for r in log)
-    print("wall %.1f ms; device span of the tasks %.1f ms; H2D %.2f GB, D2H %.2f GB; %d tasks gated on inputs" % (
-        wall, (ends - d0) / 1e6, (s1.input_tx_bytes - s0.input_tx_bytes) / 1e9, (s1.output_tx_bytes - s0.output_tx_bytes) / 1e9,
-        s1.gated_tasks - s0.gated_tasks))
+    print("wall %.1f ms (submit %.1f ms, drive setup %.1f ms); device span of the tasks %.1f ms; H2D %.2f GB, D2H %.2f GB;"
+          " %d tasks gated on inputs" % (
+              wall, sub, (s1.host_ns_drive_setup - s0.host_ns_drive_setup) / 1e6, (ends - d0) / 1e6,
+              (s1.input_tx_bytes - s0.input_tx_bytes) / 1e9, (s1.output_tx_bytes - s0.output_tx_bytes) / 1e9,
+              s1.gated_tasks - s0.gated_tasks))
     for _ in range(2):
         wl.reset()
         torch.cuda.synchronize()
