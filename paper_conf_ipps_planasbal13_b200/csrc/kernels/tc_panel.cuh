@@ -182,6 +182,29 @@ __device__ __forceinline__ void tmem_st16_issue(uint32_t taddr, const float (&v)
         : "memory");
 }
 __device__ __forceinline__ void tmem_wait_st() { asm volatile("tcgen05.wait::st.sync.aligned;" ::: "memory"); }
+// POTRF operand images (tc_potrf): per row block and 32-wide k-block the split big / small
+// values in two SW64 halves (16 k each, the layout of the cross-sub-block update operands),
+// bulk-stored from shared memory by the epilogue, bulk-copied into a stage by the producers
+constexpr int kImgHalf = BM * 64;          // 8 KB: 128 rows x 16 fp32
+constexpr int kImgKb = 4 * kImgHalf;       // 32 KB: big (2 halves) + small (2 halves)
+__device__ __forceinline__ void img_expect_tx(uint64_t *bar, uint32_t bytes)
+{
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes) : "memory");
+}
+__device__ __forceinline__ void img_g2s(uint32_t dst, const void *src, uint32_t bytes, uint64_t *bar)
+{
+    asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(dst),
+                 "l"(src), "r"(bytes), "r"(smem_u32(bar))
+                 : "memory");
+}
+__device__ __forceinline__ void img_s2g(void *dst, uint32_t src, uint32_t bytes)
+{
+    asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;" ::"l"(dst), "r"(src), "r"(bytes) : "memory");
+}
+__device__ __forceinline__ void img_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
+__device__ __forceinline__ void img_wait_read() { asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory"); }
+__device__ __forceinline__ void img_wait_all() { asm volatile("cp.async.bulk.wait_group 0;" ::: "memory"); }
+__device__ __forceinline__ void fence_proxy_async_global() { asm volatile("fence.proxy.async.global;" ::: "memory"); }
 __device__ __forceinline__ void bar_epi() { asm volatile("bar.sync 2, 128;" ::: "memory"); }
 // UMMA shared-memory descriptor, K-major SWIZZLE_64B (layout 4): 64-byte rows, 8-row atoms of
 // 512 B (SBO), version 1 — the cross-sub-block update operands (16 fp32 of K per row)
@@ -199,7 +222,7 @@ __device__ __forceinline__ uint64_t desc_sw64(uint32_t saddr)
 template <bool POTRF>
 __global__ void __launch_bounds__(PTHREADS, 1)
 tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int k_base, int *info,
-                unsigned long long launch_id, int overlap, int64_t lbs, int64_t xbs, TaskCtx ctx)
+                unsigned long long launch_id, int overlap, int64_t lbs, int64_t xbs, TaskCtx ctx, uint8_t *img)
 {
     ctx_begin(ctx);
     L += blockIdx.y * lbs;   // TRSM batch (tc_trsm_batched): independent problems along y
@@ -236,13 +259,13 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
     const unsigned long long tag = launch_id << 8;
     if (threadIdx.x == 0) {
         for (int s = 0; s < STAGES; s++) {
-            mbar_init(&full[s], NP / 32);
+            mbar_init(&full[s], img ? 1 : NP / 32);   // images: one expect_tx arrival + the bytes
             mbar_init(&empty[s], 1);
         }
         mbar_init(&accf[0], 1);
         mbar_init(&accf[1], 1);
         mbar_init(xdone, 4);
-        mbar_init(xacc, 1);
+        mbar_init(xacc, 2);   // per use: the MMA commit (or a plain arrival) + the image store's read
         mbar_init(&bfull[0], 4);
         mbar_init(&bfull[1], 4);
         mbar_init(pstart, 1);
@@ -350,25 +373,39 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     rb[p] = (c0 + row < n) ? (POTRF ? ld_f4_cg(src) : __ldg(reinterpret_cast<const float4 *>(src))) : z4;
                 }
             };
-            auto produce = [&](float4 (&ra)[APER], float4 (&rb)[BPER]) {
+            auto produce = [&](float4 (&ra)[APER], float4 (&rb)[BPER], int kb) {
                 const int s = gkb % STAGES;
-                if (gkb >= STAGES) mbar_wait(&empty[s], ((gkb / STAGES) - 1) & 1);
                 uint8_t *st = smem + s * G::STAGE;
-                uint8_t *a_big = st, *a_small = st + G::A_BYTES;
-                uint8_t *b_big = st + 2 * G::A_BYTES, *b_small = b_big + G::B_BYTES;
+                if (img) {
+                    // POTRF: the k-block's split operands exist as images (stored by the rows'
+                    // owners when they solved them): two bulk copies, no loads / splits here
+                    ensure(kb);
+                    if (t == 0) {
+                        if (gkb >= STAGES) mbar_wait(&empty[s], ((gkb / STAGES) - 1) & 1);
+                        fence_proxy_async_global();
+                        const int nkb = n / BK;
+                        img_expect_tx(&full[s], 2 * kImgKb);
+                        img_g2s(smem_u32(st), img + ((size_t)blockIdx.x * nkb + kb) * kImgKb, kImgKb, &full[s]);
+                        img_g2s(smem_u32(st) + kImgKb, img + ((size_t)J * nkb + kb) * kImgKb, kImgKb, &full[s]);
+                    }
+                } else {
+                    if (gkb >= STAGES) mbar_wait(&empty[s], ((gkb / STAGES) - 1) & 1);
+                    uint8_t *a_big = st, *a_small = st + G::A_BYTES;
+                    uint8_t *b_big = st + 2 * G::A_BYTES, *b_small = b_big + G::B_BYTES;
 #pragma unroll
-                for (int p = 0; p < APER; p++) {
-                    const int f = t + p * NP, row = f >> 3, c = f & 7;
-                    store_split(a_big, a_small, kmaj_off(row, c), ra[p]);
-                }
+                    for (int p = 0; p < APER; p++) {
+                        const int f = t + p * NP, row = f >> 3, c = f & 7;
+                        store_split(a_big, a_small, kmaj_off(row, c), ra[p]);
+                    }
 #pragma unroll
-                for (int p = 0; p < BPER; p++) {
-                    const int f = t + p * NP, row = f >> 3, c = f & 7;
-                    store_split(b_big, b_small, kmaj_off(row, c), rb[p]);
+                    for (int p = 0; p < BPER; p++) {
+                        const int f = t + p * NP, row = f >> 3, c = f & 7;
+                        store_split(b_big, b_small, kmaj_off(row, c), rb[p]);
+                    }
+                    fence_proxy_async();
+                    __syncwarp();
+                    if (lane == 0) mbar_arrive(&full[s]);   // one release-arrive per producer warp
                 }
-                fence_proxy_async();
-                __syncwarp();
-                if (lane == 0) mbar_arrive(&full[s]);   // one release-arrive per producer warp
                 if (warp == 0) {
                     // MMA issue: all four producer warps have filled stage s
                     mbar_wait(&full[s], (gkb / STAGES) & 1);
@@ -378,9 +415,16 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                         const uint32_t bb = ab + 2 * G::A_BYTES, bs = bb + G::B_BYTES;
 #pragma unroll
                         for (int kk = 0; kk < BK / 8; kk++) {
-                            const uint32_t o = kk * 32;
-                            const uint64_t dAb = make_desc(ab + o, 16, 1024), dAs = make_desc(as + o, 16, 1024);
-                            const uint64_t dBb = make_desc(bb + o, 16, 1024), dBs = make_desc(bs + o, 16, 1024);
+                            uint64_t dAb, dAs, dBb, dBs;
+                            if (img) {   // two SW64 halves of 16 k per part
+                                const uint32_t o = (uint32_t)(kk >> 1) * kImgHalf + (uint32_t)(kk & 1) * 32;
+                                dAb = desc_sw64(ab + o), dAs = desc_sw64(as + o);
+                                dBb = desc_sw64(bb + o), dBs = desc_sw64(bs + o);
+                            } else {
+                                const uint32_t o = kk * 32;
+                                dAb = make_desc(ab + o, 16, 1024), dAs = make_desc(as + o, 16, 1024);
+                                dBb = make_desc(bb + o, 16, 1024), dBs = make_desc(bs + o, 16, 1024);
+                            }
                             const uint32_t first = (kbp == 0 && kk == 0) ? 0u : 1u;
                             mma_tf32(dt, dAb, dBb, idesc, first);
                             mma_tf32(dt, dAb, dBs, idesc, 1u);
@@ -399,14 +443,18 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 gkb++;
             };
             float4 ra0[APER], rb0[BPER], ra1[APER], rb1[BPER];
-            load(ra0, rb0, 0);
-            if (nk > 1) load(ra1, rb1, 1);
-            for (int kb = 0; kb < nk; kb += 2) {
-                produce(ra0, rb0);
-                if (kb + 2 < nk) load(ra0, rb0, kb + 2);
-                if (kb + 1 < nk) {
-                    produce(ra1, rb1);
-                    if (kb + 3 < nk) load(ra1, rb1, kb + 3);
+            if (img) {
+                for (int kb = 0; kb < nk; kb++) produce(ra0, rb0, kb);
+            } else {
+                load(ra0, rb0, 0);
+                if (nk > 1) load(ra1, rb1, 1);
+                for (int kb = 0; kb < nk; kb += 2) {
+                    produce(ra0, rb0, kb);
+                    if (kb + 2 < nk) load(ra0, rb0, kb + 2);
+                    if (kb + 1 < nk) {
+                        produce(ra1, rb1, kb + 1);
+                        if (kb + 3 < nk) load(ra1, rb1, kb + 3);
+                    }
                 }
             }
             if (feed && J == fpanel) stage_b(J);   // (no k-block reached kb_new)
@@ -568,7 +616,8 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 // XS area (SW64 K-major: A = the 128 rows' 16 solved values, B = rows of L_JJ)
                 if (e == 0) PANEL_T(J, 6 + 2 * sb);
                 const bool feed_j = feed && J + 1 == fpanel;
-                if (sb + 1 < nsb || feed_j) {
+                const bool need_img = img && !factor;   // operand image of a left-of-diagonal panel
+                if (sb + 1 < nsb || feed_j || need_img) {
                     const int nb = (nsb - sb - 1) * PSB;   // later columns (a multiple of 16)
                     {   // A: this row's values, split big / small
                         const uint32_t ra = (uint32_t)e * 64u;
@@ -594,6 +643,13 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                     if (e == 0) {
                         tc_fence_after();
                         const uint32_t ab = smem_u32(xs_ab), as = smem_u32(xs_as), bb = smem_u32(xs_bb), bs = smem_u32(xs_bs);
+                        if (need_img) {   // the staged split x block is the image's half sb & 1
+                            const int nkb = n / BK;
+                            uint8_t *ib = img + ((size_t)blockIdx.x * nkb + (c0 + sb * PSB) / BK) * kImgKb + (sb & 1) * kImgHalf;
+                            img_s2g(ib, ab, kImgHalf);
+                            img_s2g(ib + 2 * kImgHalf, as, kImgHalf);
+                            img_commit();
+                        }
                         if (sb + 1 < nsb) {
                             const uint32_t idesc = make_idesc(BM, nb, false, false);
                             const uint32_t d = tmem + (uint32_t)((J & 1) * P + (sb + 1) * PSB);
@@ -624,7 +680,10 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                                 mma_tf32(d, desc_sw64(as + o), desc_sw64(ab + o), idesc, 1u);
                             }
                         }
-                        mma_commit(xacc);
+                        if (sb + 1 < nsb || feed_j) mma_commit(xacc);
+                        else mbar_arrive(xacc);
+                        if (need_img) img_wait_read();   // the staged block may be overwritten
+                        mbar_arrive(xacc);
                     }
                     mbar_wait(xacc, xacc_par);
                     xacc_par ^= 1u;
@@ -633,6 +692,10 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
                 if (e == 0) PANEL_T(J, 7 + 2 * sb);
             }
             if (e == 0) PANEL_T(J, 3);
+            if (img && !factor && e == 0) {   // the panel's images written before xdone / the flag
+                img_wait_all();
+                fence_proxy_async_global();
+            }
             // panel J of these rows: visible at L2 (own producers, other CTAs), TMEM reads done
             __threadfence();
             tc_fence_before();
@@ -657,14 +720,17 @@ tc_panel_kernel(int rows, int n, const float *L, int ldl, float *X, int ldx, int
 // kernel option bits (measurement switches): bit 0 — MMA of panel J+1 overlapped with the
 // solve of panel J (default; VS_PANEL_OVERLAP=0 serialises them); bit 1 — the diagonal CTA's
 // dry pass of the factor code (default; VS_PANEL_WARM=0 disables); bit 2 — POTRF feed of the
-// factor panel's accumulator by the previous panel's solve (default; VS_PANEL_FEED=0 disables)
+// factor panel's accumulator by the previous panel's solve (default; VS_PANEL_FEED=0 disables);
+// bit 3 — POTRF operand images (default; VS_PANEL_IMG=0: the producers load and split)
 inline int panel_overlap()
 {
     static const int v = [] {
         const char *e = getenv("VS_PANEL_OVERLAP");
         const char *w = getenv("VS_PANEL_WARM");
         const char *f = getenv("VS_PANEL_FEED");
-        return (e ? (atoi(e) ? 1 : 0) : 1) | ((w ? (atoi(w) ? 1 : 0) : 1) << 1) | ((f ? (atoi(f) ? 1 : 0) : 1) << 2);
+        const char *im = getenv("VS_PANEL_IMG");
+        return (e ? (atoi(e) ? 1 : 0) : 1) | ((w ? (atoi(w) ? 1 : 0) : 1) << 1) | ((f ? (atoi(f) ? 1 : 0) : 1) << 2) |
+               ((im ? (atoi(im) ? 1 : 0) : 1) << 3);
     }();
     return v;
 }
@@ -690,7 +756,7 @@ inline int tc_trsm(int rows, int n, const float *L, int ldl, float *X, int ldx, 
     panel_attr<false>();
     count_launch();
     tc_panel_kernel<false><<<(rows + BM - 1) / BM, PTHREADS, PanelCfg::SMEM, s>>>(rows, n, L, ldl, X, ldx, 0, nullptr,
-                                                                                  0ull, panel_overlap(), 0, 0, ctx);
+                                                                                  0ull, panel_overlap(), 0, 0, ctx, nullptr);
     return 0;
 }
 
@@ -703,7 +769,7 @@ inline int tc_trsm_batched(int count, int rows, int n, const float *L, int ldl, 
     panel_attr<false>();
     count_launch();
     tc_panel_kernel<false><<<dim3((rows + BM - 1) / BM, count), PTHREADS, PanelCfg::SMEM, s>>>(
-        rows, n, L, ldl, X, ldx, 0, nullptr, 0ull, panel_overlap(), lbs, xbs, TaskCtx());
+        rows, n, L, ldl, X, ldx, 0, nullptr, 0ull, panel_overlap(), lbs, xbs, TaskCtx(), nullptr);
     return 0;
 }
 
@@ -740,8 +806,31 @@ inline int tc_potrf(int n, float *A, int lda, int k_base, int *info, cudaStream_
     panel_attr<true>();
     count_launch();
     const int grid = (n + BM - 1) / BM;
+    // operand images (option bit 3, VS_PANEL_IMG): stream-ordered scratch from the device's
+    // default memory pool (its release threshold raised once, so the pool keeps the memory)
+    uint8_t *img = nullptr;
+    if (panel_overlap() & 8) {
+        static bool pool_set[64] = {};
+        int dev = 0;
+        cudaGetDevice(&dev);
+        cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+        cudaStreamIsCapturing(s, &cs);
+        if (!pool_set[dev & 63] && cs == cudaStreamCaptureStatusNone) {
+            cudaMemPool_t pool;
+            if (cudaDeviceGetDefaultMemPool(&pool, dev) == cudaSuccess) {
+                unsigned long long thr = ~0ull;
+                cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr);
+            }
+            pool_set[dev & 63] = true;
+        }
+        if (cudaMallocAsync((void **)&img, (size_t)grid * (n / BK) * kImgKb, s) != cudaSuccess) {
+            cudaGetLastError();
+            img = nullptr;   // the loads-and-splits producers
+        }
+    }
     tc_panel_kernel<true><<<grid, PTHREADS, PanelCfg::SMEM, s>>>(n, n, A, lda, A, lda, k_base, info, id,
-                                                                 panel_overlap(), 0, 0, ctx);
+                                                                 panel_overlap(), 0, 0, ctx, img);
+    if (img) cudaFreeAsync(img, s);
     return 0;
 }
 

@@ -183,8 +183,10 @@ def test_wait_noflush_and_wait_on_without_flush(gpu):
 
 def test_wait_on_while_other_tasks_run(gpu):
     """taskwait on(d) returns once d's last writer is done and d is valid at home, without
-    waiting for the rest of the graph; the rest completes at the next wait."""
-    N, b = 1024, 256
+    waiting for the rest of the graph; the rest completes at the next wait.  512 tasks, so that
+    C_00's 8-task chain (submitted first) cannot be observed only after the whole graph ran
+    (with 64 tasks the GPU occasionally finished them all before the host's first poll)."""
+    N, b = 2048, 256
     nt = N // b
     rt = vs.Runtime(vs.vs_config_default(lam=1, slots_per_gpu=2))
     types, (A, B), (tA, tB, tC), (ia, ib, ic) = _host_matmul(rt, N, b, 41)

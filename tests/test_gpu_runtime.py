@@ -149,6 +149,36 @@ def test_staged_host_batch_matmul_and_cholesky(gpu, stage):
     rt.close()
 
 
+def test_depend_on_event_orders_the_batch_after_the_callers_stream(gpu):
+    # vs_depend_on_event: the inputs are written on the caller's stream behind a long sleep and
+    # the batch is submitted without any host synchronisation; its kernels must still see them
+    import torch
+
+    import bench
+    rt = vs.Runtime(bench.bench_config(vs, lam=1, slots_per_gpu=4))
+    mask = (1 << vs.VS_V_TC_3XTF32) | (1 << vs.VS_V_TC_3XF16)
+    types = rt.vs_register_builtins(vs.VS_F32, mask)
+    N, b = 1024, 256
+    A, B = vsgen.uniform(91, N, N), vsgen.uniform(92, N, N)
+    src = [_tiles_dev(x, b) for x in (A, B)]
+    tA, tB, tC = (torch.zeros((N // b, N // b, b, b), device="cuda") for _ in range(3))
+    ia, ib, ic = (_register_tiles(rt, t, 0) for t in (tA, tB, tC))
+    s = torch.cuda.Stream()
+    with torch.cuda.stream(s):
+        torch.cuda._sleep(200_000_000)     # ~0.1 s of GPU time before the inputs exist
+        tA.copy_(src[0])
+        tB.copy_(src[1])
+        ev = torch.cuda.Event()
+        ev.record(s)
+    rt.vs_depend_on_event(ev)
+    rt.vs_app_matmul(types[vs.VS_T_MATMUL], 4, 4, 4, ia, ib, ic)
+    rt.vs_wait_all()
+    torch.cuda.synchronize()
+    C = vsgen.from_tiles(tC.cpu().numpy())
+    assert oracle.relF(C, oracle.matmul(A, B)) <= 1e-5
+    rt.close()
+
+
 def test_equally_critical_chains_run_concurrently(gpu):
     # R33: in the bench configuration (bottom-level priority, critical-path streams) a lone
     # matmul has 16 equally critical k-chains; they must run side by side, not queue on the
