@@ -809,7 +809,7 @@ inline int tc_potrf(int n, float *A, int lda, int k_base, int *info, cudaStream_
     // operand images (option bit 3, VS_PANEL_IMG): stream-ordered scratch from the device's
     // default memory pool (its release threshold raised once, so the pool keeps the memory)
     uint8_t *img = nullptr;
-    if (panel_overlap() & 8) {
+    if ((panel_overlap() & 8) && n >= 1024) {   // b = 512: 190 vs 183 us with images (4 panels)
         static bool pool_set[64] = {};
         int dev = 0;
         cudaGetDevice(&dev);
