@@ -22,6 +22,16 @@ namespace vsk {
 namespace tc {
 
 constexpr int kInvH0 = 64;
+// first block size of the doubling (VS_INV_H0 = 64 | 128, measurement switch): 128 when it
+// divides n — one batched 128-wide substitution replaces the 64-wide one and the first level
+inline int inv_h0(int n)
+{
+    static const int v = [] {
+        const char *e = getenv("VS_INV_H0");
+        return e ? atoi(e) : 128;
+    }();
+    return (v == 128 && n % 128 == 0) ? 128 : kInvH0;
+}
 
 // scratch floats needed by tc_inv_lt for an n x n tile
 inline size_t inv_lt_scratch(int n) { return (size_t)n * n / 4 + 64; }
@@ -31,11 +41,10 @@ inline int tc_inv_lt(int n, const float *L, int ldl, float *X, int ldx, float *T
 {
     if (n <= 0) return 0;
     if (n % kInvH0) return -1;
-    const int nb = n / kInvH0;
-    if (tc_trsm_batched(nb, kInvH0, kInvH0, L, ldl, (int64_t)kInvH0 * (ldl + 1), X, ldx, (int64_t)kInvH0 * (ldx + 1),
-                        s))
-        return -1;
-    for (int h = kInvH0; h < n; h *= 2) {
+    const int h0 = inv_h0(n);
+    const int nb = n / h0;
+    if (tc_trsm_batched(nb, h0, h0, L, ldl, (int64_t)h0 * (ldl + 1), X, ldx, (int64_t)h0 * (ldx + 1), s)) return -1;
+    for (int h = h0; h < n; h *= 2) {
         const int full = n / (2 * h), rem = n - full * 2 * h;
         auto pairs = [&](int o, int h2, int count) {
             const int64_t xs = (int64_t)2 * h * (ldx + 1), ls = (int64_t)2 * h * (ldl + 1);

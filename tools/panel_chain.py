@@ -12,3 +12,8 @@ for J in range(0, 7):
     print(J, 'factor %.1f | flag+%.1f staged+%.1f acc+%.1f solved+%.1f nextacc+%.1f' % row)
     print('   solve sub-blocks of CTA J+1 (from staged):', ' '.join('%.1f' % ((tr[c, J, i] - tr[c, J, 1]) / 1e3) for i in range(6, 22, 2)))
 print('potrf span (CTA0 accready/first -> CTA7 solved): %.1f us' % ((tr[7, 7, 3] - tr[1, 0, 0]) / 1e3))
+print('factor CTA J, panel J: per 16-column sub-block (from accready): solved | cross update done; [22] x = b - acc, [23] solve done')
+for J in range(1, 8):
+    a = tr[J, J, 2]
+    print(J, ' '.join('%.1f|%.1f' % ((tr[J, J, 6 + 2 * sb] - a) / 1e3, (tr[J, J, 7 + 2 * sb] - a) / 1e3) for sb in range(8)),
+          ' [22] %.1f [23] %.1f' % ((tr[J, J, 22] - a) / 1e3, (tr[J, J, 23] - a) / 1e3))
