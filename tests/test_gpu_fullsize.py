@@ -83,3 +83,49 @@ def test_fullsize_bench_configuration(gpu):
     st = rt.vs_stats()
     assert st.tasks_completed == 2 * (4096 + 5984)
     rt.close()
+
+
+def test_fullsize_host_homed_transfer_ordered(gpu):
+    """The e2e configuration of bench.py: the same cfg3 + cfg4 step with every tile homed in
+    pinned host memory, moved by the runtime in the transfer-ordered drive (R39) and written back
+    home; sampled matmul rows and the leading 2048 block of the factor against the oracle."""
+    import torch
+
+    import bench
+    rt = vs.Runtime(bench.bench_config(vs))
+    wl = bench.Workload(rt, host=True)
+    wl.step()
+    s0 = rt.vs_stats()
+    wl.step()          # restores and invalidates the inputs, then the timed-like step
+    s1 = rt.vs_stats()
+    torch.cuda.synchronize()
+    assert s1.gated_tasks > s0.gated_tasks                   # the staged drive ran
+    n_in = 3 * (bench.MM_N // bench.MM_B) ** 2 + (bench.CH_N // bench.CH_B) * (bench.CH_N // bench.CH_B + 1) // 2
+    assert s1.input_tx_bytes - s0.input_tx_bytes == n_in * bench.MM_B * bench.MM_B * 4
+    N, b = bench.MM_N, bench.MM_B
+    nt = N // b
+    Bfull = vsgen.uniform(bench.SEED_MM + 1000, N, N)
+    for r in (0, 5000, 16383):
+        a = vsgen.uniform_idx(bench.SEED_MM, np.arange(r * N, (r + 1) * N, dtype=np.uint64)).astype(np.float32)
+        ref = oracle.matmul(a[None, :], Bfull)[0]
+        got = wl.C.view(nt, nt, b, b)[r // b, :, r % b, :].reshape(-1).numpy()
+        assert oracle.relF(got, ref) <= 1e-5, r
+    del Bfull
+    Nc, bc = bench.CH_N, bench.CH_B
+    k = 2048
+    host = wl.S.numpy()                                        # lower tiles in row order
+    L = np.zeros((k, k), np.float32)
+    t = 0
+    for i in range(Nc // bc):
+        for j in range(i + 1):
+            if i * bc < k and j * bc < k:
+                L[i * bc:(i + 1) * bc, j * bc:(j + 1) * bc] = host[t]
+            t += 1
+    L = np.tril(L)
+    r_ = np.arange(k, dtype=np.uint64)[:, None]
+    c_ = np.arange(k, dtype=np.uint64)[None, :]
+    S = vsgen.uniform_idx(bench.SEED_CH, np.maximum(r_, c_) * np.uint64(Nc) + np.minimum(r_, c_))
+    S[np.arange(k), np.arange(k)] += vsgen.spd_alpha(Nc)
+    Lk, info = oracle.cholesky(S.astype(np.float32))
+    assert info == 0 and oracle.relF(L, Lk) <= 1e-5
+    rt.close()
