@@ -716,7 +716,14 @@ def main():
             "operand_forms_per_step": int((st1.forms_built - st0.forms_built) / args.steps),
             "device_tx_bytes_per_step": int((st1.device_tx_bytes - st0.device_tx_bytes) / args.steps),
             "host_us_per_task": {k: round((getattr(st1, "host_ns_" + k) - getattr(st0, "host_ns_" + k)) / 1e3 / max(1, len(log)), 3)
-                                 for k in ("decide", "issue", "launch", "deps", "poll", "vevent", "flush")},
+                                 for k in ("decide", "issue", "launch", "deps", "poll", "poll_idle", "vevent", "flush")},
+            # host time per task spent doing work: polls that found completions (they include the
+            # decisions and issues those completions trigger; launch and deps are parts of issue)
+            # + grouped launches from the loop; the rest of the drive loop waits on the GPU
+            "host_busy_us_per_task": round(sum(getattr(st1, "host_ns_" + k) - getattr(st0, "host_ns_" + k)
+                                               for k in ("poll", "vevent", "flush"))
+                                           / 1e3 / max(1, len(log)) -
+                                           (st1.host_ns_poll_idle - st0.host_ns_poll_idle) / 1e3 / max(1, len(log)), 3),
             "host_idle_loops_per_task": round((st1.host_idle_loops - st0.host_idle_loops) / max(1, len(log)), 2),
             "host_us_per_group_launch": round((st1.host_ns_group_launch - st0.host_ns_group_launch) / 1e3 /
                                               max(1, st1.group_launches - st0.group_launches), 2),

@@ -319,6 +319,8 @@ typedef struct {
     int64_t host_ns_drive_setup; /* host time from entering a wait's drive to its first
                                  decisions issued (dependence tracker upload, bottom levels,
                                  transfer plan) */
+    int64_t host_ns_poll_idle;   /* part of host_ns_poll spent in polls that found no completed
+                                 task (the host waiting on the GPU) */
 } vs_stats_t;
 int vs_stats(vs_rt rt, vs_stats_t *out);
 

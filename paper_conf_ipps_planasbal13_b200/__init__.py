@@ -56,7 +56,7 @@ class vs_stats_t(Structure):
         "tasks_submitted", "tasks_completed", "decisions", "input_tx_bytes", "output_tx_bytes", "device_tx_bytes",
         "n_groups", "error_task", "error_info", "host_ns_decide", "host_ns_issue", "virtual_now_ns",
         "kernel_launches", "tracker", "forms_built", "host_ns_poll", "host_ns_launch", "host_ns_deps", "host_loops", "host_ns_vevent", "host_ns_flush",
-        "host_idle_loops", "device_released", "host_ns_group_launch", "group_launches", "gated_tasks", "host_ns_drive_setup")]
+        "host_idle_loops", "device_released", "host_ns_group_launch", "group_launches", "gated_tasks", "host_ns_drive_setup", "host_ns_poll_idle")]
 
 
 class vs_group_stat_t(Structure):
