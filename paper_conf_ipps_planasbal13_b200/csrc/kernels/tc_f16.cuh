@@ -41,8 +41,7 @@
 //               accumulator, tcgen05.ld 32-column chunks -> padded per-warp smem block (the
 //               stage buffers are free once acc_full fired), then row by row coalesced:
 //               C = C_in + acc * 2^-eA(i) * 2^-eB(j) in fp32 round-to-nearest (C_in read
-//               from global here; each epilogue thread prefetches its C row into L2 at
-//               kernel start).
+//               from global here; an L2 prefetch of it at kernel start measured slower).
 // LOWER (syrk): tiles strictly above the diagonal exit; diagonal tiles store only j <= i.
 #pragma once
 #include <cuda_fp16.h>
@@ -287,10 +286,6 @@ __device__ __forceinline__ uint32_t cluster_ctarank()
     return r;
 }
 
-__device__ __forceinline__ void prefetch_l2(const void *p, uint32_t bytes)
-{
-    asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(p), "r"(bytes) : "memory");
-}
 
 // UMMA shared-memory descriptor, K-major SWIZZLE_64B (layout type 4): rows of 64 B, 8-row
 // atoms of 512 B (SBO), LBO = 16 B (ignored for swizzled K-major), version 1.
@@ -503,13 +498,9 @@ __global__ void __launch_bounds__(NTHREADS, 1) tcf_gemm_kernel(const __grid_cons
         const float *sav = tk.sa + m0;
         const float4 sb = __ldg(reinterpret_cast<const float4 *>(tk.sb + n0 + ccol));
         const bool BETA0 = (tk.flags >> 2) & 1;   // C = s A B'^T (C_in not read)
-        if (!BETA0 && !ghost) {   // C_in into L2 while the main loop runs (LSU prefetches: bulk prefetches
-            // would occupy the TMA unit that feeds the operands): thread t -> tile row t, its 1 KB
-            const int r = threadIdx.x - 64;
-            if (m0 + r < M)
-                for (int c = 0; c < min(BT, N - n0); c += 32)
-                    asm volatile("prefetch.global.L2 [%0];" ::"l"(C + (int64_t)(m0 + r) * ldc + n0 + c));
-        }
+        // (no L2 prefetch of C_in during the main loop: measured in the bench with and without,
+        // interleaved, 303-307 vs 308-310 TFLOP/s — the 256 KB per CTA issued at kernel start
+        // competes with the operand streams for L2 and is partly evicted before the epilogue)
         if (warp == 2 && lane == 0) TCF_T(5);
         mbar_wait(acc_full, 0);
         tc_fence_after();
