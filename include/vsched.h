@@ -207,7 +207,7 @@ typedef struct {
  * VS_GROUP(=tasks per grouped launch), VS_GROUP_US, VS_STAGE(=n).  Runtime options outside vs_config:
  * VS_TRACKER(=events|memops) dependence tracker on one GPU, VS_GROUP_DIST(=0|1, default 1)
  * grouped launches in a multi-rank job, VS_PREFETCH(=n, default 0) input-prefetch window on one
- * GPU, VS_TCF_PAIR(=0|1, default 1) CTA-pair variant of the tc_3xf16 GEMM. */
+ * GPU, VS_TCF_PAIR(=0|1, default 0) CTA-pair variant of the tc_3xf16 GEMM. */
 void vs_config_default(vs_config *cfg);
 
 /* Create a runtime.  *out receives an opaque handle owning scheduler state, DAG,

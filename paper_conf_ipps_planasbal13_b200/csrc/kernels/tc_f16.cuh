@@ -602,9 +602,12 @@ inline int split_cols(const float *X, int K, int R, int ld, void *out, cudaStrea
 // CTA-pair (A multicast) variant of the GEMM: on unless VS_TCF_PAIR=0
 inline bool tcf_pair()
 {
+    // CTA pairs with A multicast (VS_TCF_PAIR=1): measured equal to single CTAs in session 3 and
+    // 1.2 % slower (308.4-309.0 vs 311.2-312.9 TFLOP/s interleaved) once the C_in L2 prefetch was
+    // gone: single CTAs by default
     static const int v = [] {
         const char *e = getenv("VS_TCF_PAIR");
-        return e ? atoi(e) : 1;
+        return e ? atoi(e) : 0;
     }();
     return v != 0;
 }
