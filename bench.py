@@ -64,9 +64,9 @@ def bench_config(vs, **over):
     return vs.vs_config_default(**kw)
 
 
-def ncu_traffic(path=os.path.join(ROOT, "profiles", "r02_ncu_full_tcf_bench.csv")):
+def ncu_traffic(path=os.path.join(ROOT, "profiles", "r02s4_ncu_full_tcf_bench.csv")):
     """dram__bytes_read.sum + dram__bytes_write.sum of the committed ncu --set full capture of
-    one steady-state tcf_gemm_kernel<24,1> launch inside the bench (8 tasks, 128 CTAs; bytes per
+    one steady-state tcf_gemm_kernel<24,0> launch inside the bench (8 tasks, 128 CTAs; bytes per
     launch), or None."""
     import csv
     scale = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}
@@ -354,9 +354,10 @@ def roofline(log, groups, ms, world, launch_of=None):
     roof = {"bound": bound, "kernel": dom, "tasks": d["n"], "achieved": round(achieved, 2), "peak": round(peak, 1),
             "unit": "TFLOP/s", "frac": round(achieved / peak, 4), "traffic": traffic,
             "traffic_note": ("DRAM bytes of one captured steady-state launch (ncu --set full, "
-                             "profiles/r02_ncu_full_tcf_bench.csv: tcf_gemm_kernel<24,1>, 8 MATMUL/GEMM_NT tasks, "
+                             "profiles/r02s4_ncu_full_tcf_bench.csv: tcf_gemm_kernel<24,0>, 8 MATMUL/GEMM_NT tasks, "
                              "128 CTAs; algorithmic reads 8 x (A form 4 MiB + B form 4 MiB + C 4 MiB) = 100.7 MB, "
-                             "writes 33.6 MB, most of which leave L2 after the kernel)") if traffic else None,
+                             "writes 33.6 MB: operand forms shared with earlier launches hit L2, the C writes leave "
+                             "L2 after the kernel)") if traffic else None,
             "per_launch": per_launch,
             "peak_source": src,
             "how": "hardware MMA flops (3x the algorithmic flops of its tasks: 2b^3 matmul/gemm, b^3 syrk/trsm) of "
